@@ -1,0 +1,220 @@
+"""Pins of the CPU oracle (oracle/conv2d_oracle.c) against things other than itself.
+
+Closed forms (impulse, delta filter, K=1, constant input, box filter vs summed-area table), exactness
+with integer data, textbook/library routines on tiny inputs (scipy.signal.correlate2d, float64
+torch.nn.functional.conv2d), invariants (linearity, separability, channel decomposition, NaN
+receptive field), and the sampled/row-range entry points against the full computation.
+"""
+import numpy as np
+import pytest
+import scipy.signal
+import torch
+
+import oracle
+from gen import synth
+
+RNG = np.random.default_rng(20200914)
+
+
+def _img(H, W, dist="sym", seed=1):
+    return synth.fill_np(seed, synth.TAG_INPUT, (H, W), dist)
+
+
+def _flt(K, dist="rand", seed=2):
+    return synth.make_filter(seed, K, dist)[0, 0]
+
+
+# ---------------------------------------------------------------- closed forms (bitwise)
+@pytest.mark.parametrize("K", [1, 2, 3, 5, 8, 15])
+def test_impulse_input_gives_filter(K):
+    """in = e_(r0,c0) => out[y][x] = f[r0-y][c0-x] inside the range, else 0 (orientation: no flip)."""
+    H, W = K + 9, K + 7
+    f = _flt(K, "rand", seed=K)
+    for (r0, c0) in [(0, 0), (K - 1, K - 1), (H // 2, W // 3), (H - 1, W - 1)]:
+        img = np.zeros((H, W), np.float32)
+        img[r0, c0] = 1.0
+        out, _, _ = oracle.conv2d_single(img, f)
+        exp = np.zeros_like(out)
+        for y in range(out.shape[0]):
+            for x in range(out.shape[1]):
+                i, j = r0 - y, c0 - x
+                if 0 <= i < K and 0 <= j < K:
+                    exp[y, x] = f[i, j]
+        assert np.array_equal(out.view(np.uint32), exp.view(np.uint32))
+
+
+@pytest.mark.parametrize("K", [1, 3, 4, 7, 15])
+def test_delta_filter_is_shift(K):
+    """f = e_(i0,j0) => out[y][x] = in[y+i0][x+j0] (BASELINE.json north_star closed form)."""
+    H, W = 2 * K + 5, 3 * K + 2
+    img = _img(H, W, "img", seed=K)
+    Ho, Wo = H - K + 1, W - K + 1
+    for (i0, j0) in {(0, 0), (K - 1, 0), (0, K - 1), (K // 2, K // 2), (K - 1, K - 1)}:
+        f = np.zeros((K, K), np.float32)
+        f[i0, j0] = 1.0
+        out, _, _ = oracle.conv2d_single(img, f)
+        assert np.array_equal(out, img[i0:i0 + Ho, j0:j0 + Wo])
+
+
+def test_k1_is_correctly_rounded_scale():
+    img = _img(33, 41, "sym")
+    for w in (np.float32(0.3), np.float32(-1.7e-3), np.float32(3.0)):
+        out, _, _ = oracle.conv2d_single(img, np.array([[w]], np.float32))
+        assert np.array_equal(out, img * w)  # IEEE fp32 product = one rounding of the exact product
+
+
+@pytest.mark.parametrize("K", [2, 3, 5, 9, 15])
+def test_constant_input(K):
+    """in == c => out == c * sum(w) exactly for dyadic c and small-integer w."""
+    c = np.float32(0.75)
+    f = synth.make_filter(K, K, "int")[0, 0]
+    img = np.full((K + 6, K + 11), c, np.float32)
+    out, _, _ = oracle.conv2d_single(img, f)
+    assert (out == np.float32(float(c) * float(f.astype(np.float64).sum()))).all()
+
+
+@pytest.mark.parametrize("K", [1, 3, 6, 11, 15])
+def test_box_filter_matches_summed_area_table(K):
+    """Box filter == prefix-sum result S[y+K][x+K] - S[y][x+K] - S[y+K][x] + S[y][x] (int64)."""
+    H, W = K + 20, K + 17
+    img = _img(H, W, "int", seed=K)
+    S = np.zeros((H + 1, W + 1), np.int64)
+    S[1:, 1:] = img.astype(np.int64).cumsum(0).cumsum(1)
+    exp = S[K:, K:] - S[:-K, K:] - S[K:, :-K] + S[:-K, :-K]
+    out, _, _ = oracle.conv2d_single(img, np.ones((K, K), np.float32))
+    assert np.array_equal(out, exp.astype(np.float32))
+
+
+def test_integer_data_exact():
+    """Integer data: every partial sum is an exactly representable integer -> exact result."""
+    for K in (3, 7, 15):
+        img = _img(K + 13, K + 9, "int", seed=K)
+        f = synth.make_filter(K, K, "int")[0, 0]
+        out, bound, out64 = oracle.conv2d_single(img, f, want_f64=True)
+        ref = np.zeros(out.shape, np.int64)
+        for y in range(out.shape[0]):
+            for x in range(out.shape[1]):
+                ref[y, x] = int((img[y:y + K, x:x + K].astype(np.int64) * f.astype(np.int64)).sum())
+        assert np.array_equal(out64, ref.astype(np.float64))
+        assert np.array_equal(out, ref.astype(np.float32))
+        assert (bound >= np.abs(out64)).all()
+
+
+# ---------------------------------------------------------------- textbook / library routines
+def test_matches_scipy_correlate2d_bruteforce():
+    """Tiny inputs, K = 1..15, H, W in [K, K+6]: out64 == scipy.signal.correlate2d(valid)."""
+    for K in range(1, 16):
+        for trial in range(3):
+            H = K + int(RNG.integers(0, 7))
+            W = K + int(RNG.integers(0, 7))
+            img = RNG.standard_normal((H, W)).astype(np.float32)
+            f = RNG.standard_normal((K, K)).astype(np.float32)
+            out, bound, out64 = oracle.conv2d_single(img, f, want_f64=True)
+            ref = scipy.signal.correlate2d(img.astype(np.float64), f.astype(np.float64), mode="valid")
+            assert ref.shape == out.shape
+            assert (np.abs(out64 - ref) <= 1e-12 * bound).all()
+            assert np.array_equal(out, out64.astype(np.float32))  # exactly one rounding
+            ab = scipy.signal.correlate2d(np.abs(img.astype(np.float64)), np.abs(f.astype(np.float64)),
+                                          mode="valid")
+            assert np.allclose(bound, ab, rtol=1e-12, atol=0)
+
+
+def test_multi_matches_torch_conv2d_float64():
+    """Multi-channel oracle == float64 torch.nn.functional.conv2d (OIHW, cross-correlation)."""
+    for (N, C, F, K, H, W) in [(1, 1, 1, 3, 7, 9), (2, 3, 4, 5, 11, 8), (2, 4, 3, 7, 9, 13),
+                               (1, 2, 2, 1, 4, 4), (3, 3, 2, 15, 16, 18), (1, 4, 5, 4, 10, 6)]:
+        inp = RNG.standard_normal((N, C, H, W)).astype(np.float32)
+        w = RNG.standard_normal((F, C, K, K)).astype(np.float32)
+        out, bound, out64 = oracle.conv2d_multi(inp, w, want_f64=True)
+        ref = torch.nn.functional.conv2d(torch.from_numpy(inp).double(), torch.from_numpy(w).double())
+        assert (np.abs(out64 - ref.numpy()) <= 1e-12 * bound).all()
+        assert np.array_equal(out, out64.astype(np.float32))
+
+
+# ---------------------------------------------------------------- invariants
+def test_linearity():
+    K = 5
+    x = _img(30, 31, "sym", 1)
+    y = _img(30, 31, "sym", 2)
+    f = _flt(K)
+    a, b = 1.0, -1.0  # sym values are k/2^23 with |k| <= 2^23: x - y is exact in fp32
+    z = (a * x.astype(np.float64) + b * y.astype(np.float64)).astype(np.float32)
+    assert np.array_equal(z.astype(np.float64), a * x.astype(np.float64) + b * y.astype(np.float64))
+    _, bz, oz = oracle.conv2d_single(z, f, want_f64=True)
+    _, _, ox = oracle.conv2d_single(x, f, want_f64=True)
+    _, _, oy = oracle.conv2d_single(y, f, want_f64=True)
+    assert (np.abs(oz - (a * ox + b * oy)) <= 1e-12 * (bz + 1)).all()
+    _, _, o4 = oracle.conv2d_single(x * np.float32(4.0), f, want_f64=True)  # exact power-of-2 scale
+    assert np.array_equal(o4, 4.0 * ox)
+
+
+def test_separable_filter():
+    """f = u v^T: conv == column pass by u of the row pass by v."""
+    K = 7
+    u = RNG.standard_normal(K).astype(np.float32)
+    v = RNG.standard_normal(K).astype(np.float32)
+    f = np.outer(u.astype(np.float64), v.astype(np.float64))
+    f32 = f.astype(np.float32)
+    img = _img(40, 37, "sym")
+    _, bound, o64 = oracle.conv2d_single(img, f32, want_f64=True)
+    rows = np.stack([np.correlate(r.astype(np.float64), v.astype(np.float64), "valid") for r in img])
+    sep = np.stack([np.correlate(c, u.astype(np.float64), "valid") for c in rows.T]).T
+    # f32 = f rounded: allow the filter rounding (2^-24 relative per tap) in the comparison
+    assert (np.abs(o64 - sep) <= 1e-6 * bound).all()
+
+
+def test_multi_is_sum_over_channels_and_reduces_to_single():
+    N, C, F, K, H, W = 2, 3, 2, 4, 12, 15
+    inp = synth.fill_np(4, 1, (N, C, H, W), "sym")
+    w = synth.make_filter(4, K, "rand", F=F, C=C)
+    out, bound, out64 = oracle.conv2d_multi(inp, w, want_f64=True)
+    for n in range(N):
+        for f in range(F):
+            s = sum(oracle.conv2d_single(inp[n, c], w[f, c], want_f64=True)[2] for c in range(C))
+            assert (np.abs(out64[n, f] - s) <= 1e-12 * bound[n, f]).all()
+    o1, _, _ = oracle.conv2d_multi(inp[:1, :1], w[:1, :1])
+    s1, _, _ = oracle.conv2d_single(inp[0, 0], w[0, 0])
+    assert np.array_equal(o1[0, 0], s1)
+
+
+def test_nan_receptive_field():
+    """A NaN at (r, c) poisons exactly outputs y in [r-K+1, r], x in [c-K+1, c]."""
+    K, H, W = 5, 20, 23
+    img = _img(H, W, "img")
+    r, c = 9, 11
+    img[r, c] = np.nan
+    out, _, _ = oracle.conv2d_single(img, _flt(K))
+    mask = np.zeros(out.shape, bool)
+    mask[max(0, r - K + 1):r + 1, max(0, c - K + 1):c + 1] = True
+    assert np.array_equal(np.isnan(out), mask)
+
+
+# ---------------------------------------------------------------- entry points agree
+def test_points_and_rows_match_full():
+    K = 6
+    img = _img(50, 61, "img")
+    f = _flt(K)
+    out, bound, _ = oracle.conv2d_single(img, f)
+    ys = RNG.integers(0, out.shape[0], 200)
+    xs = RNG.integers(0, out.shape[1], 200)
+    po, pb = oracle.conv2d_single_points(img, f, ys, xs)
+    assert np.array_equal(po, out[ys, xs]) and np.array_equal(pb, bound[ys, xs])
+    ro, _, _ = oracle.conv2d_single(img, f, rows=(7, 19))
+    assert np.array_equal(ro[7:19], out[7:19])
+
+    inp = synth.fill_np(9, 1, (3, 2, 14, 17), "sym")
+    w = synth.make_filter(9, 3, "he", F=4, C=2)
+    mo, mb, _ = oracle.conv2d_multi(inp, w)
+    n, fi, y, x = (RNG.integers(0, s, 100) for s in mo.shape)
+    qo, qb = oracle.conv2d_multi_points(inp, w, n, fi, y, x)
+    assert np.array_equal(qo, mo[n, fi, y, x]) and np.array_equal(qb, mb[n, fi, y, x])
+    io, _, _ = oracle.conv2d_multi(inp, w, images=(1, 3))
+    assert np.array_equal(io[1:3], mo[1:3])
+
+
+def test_within_tolerance_helper():
+    ref = np.array([1.0, 2.0, np.nan, 0.0])
+    bound = np.array([1.0, 1.0, 1.0, 0.0])
+    assert oracle.within_tolerance(ref + [1e-6, 0, 0, 0], ref, bound).tolist() == [True, True, True, True]
+    assert not oracle.within_tolerance(ref + [2e-5, 0, 0, 0], ref, bound)[0]
+    assert not oracle.within_tolerance(ref + [0, 0, 0, 1e-30], ref, bound)[3]
