@@ -1,0 +1,101 @@
+/*
+ * conv2d.h -- C ABI of the B200 (sm_100a) direct-convolution library libconv2d.so.
+ *
+ * The operation is the one Lu, Zhang & Wang, "Optimizing GPU Memory Transactions for Convolution
+ * Operations" (IEEE Cluster 2020) accelerate: direct, stride-1, valid-mode fp32 2D convolution
+ * (cross-correlation, no filter flip), for a single-channel image (Fig. 1 P:130-203,
+ * Fig. 2 equations) and for multi-channel N x C x F convolution (Table I
+ * P:335-352, naming P:350-352). The kernels behind these calls implement the paper's column reuse
+ * (warp-shuffle exchange of overlapping input columns with static register indices, Alg. 1
+ * P:243-254) and row reuse (each loaded input row multiplied by several filter rows,
+ * Alg. 2), re-designed for sm_100a.
+ *
+ * Conventions shared by every entry point
+ *   - All tensor pointers are DEVICE pointers (global memory of the current CUDA device), owned by
+ *     the caller. The library never allocates, frees, or retains them after the call returns.
+ *   - fp32, dense, row-major: no strides, no padding; every pointer must be 4-byte aligned. Any
+ *     width and any 4-byte alignment is supported; 16-byte-aligned inputs with W % 4 == 0 take the
+ *     vectorised (LDG.128) path.
+ *   - `stream` is a cudaStream_t passed as void* (NULL = legacy default stream). Work is enqueued
+ *     asynchronously on it; there is no host synchronisation. The call is reentrant and thread-safe:
+ *     filters are staged per CTA into shared memory, there is no module-global mutable state.
+ *   - Return value: 0 when the work was enqueued. A negative CONV2D_E* code when an argument is
+ *     invalid (nothing was launched) or the launch itself failed. Asynchronous execution errors
+ *     surface at the caller's next synchronisation, as in CUDA.
+ *   - Stride 1, no padding ("valid"): Ho = H-K+1, Wo = W-K+1. Square K x K filters, 1 <= K <= 15
+ *     (R14). Every output element is written exactly once and never read.
+ *   - Arithmetic: fp32 FMA, accumulated per output in filter-row / filter-column order (multi:
+ *     filter-row, channel, filter-column). Acceptance vs the CPU oracle: |gpu - ref| <= 1e-5 *
+ *     sum|x||w| per element (BASELINE.json north_star). No fast-math, denormals preserved.
+ */
+#ifndef CONV2D_B200_H
+#define CONV2D_B200_H
+
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+#define CONV2D_OK 0
+#define CONV2D_ENULL (-1)     /* a tensor pointer is NULL */
+#define CONV2D_ESHAPE (-2)    /* H<K, W<K, N/C/F<1, K<1, or an element count above 2^62 */
+#define CONV2D_EK (-3)        /* K > 15 (K is a compile-time template parameter of the kernels) */
+#define CONV2D_EOVERLAP (-4)  /* the output range overlaps the input or the filter range */
+#define CONV2D_ECUDA (-5)     /* the kernel launch failed (cudaGetLastError after the launch) */
+#define CONV2D_EALIGN (-6)    /* a tensor pointer is not 4-byte aligned */
+
+#define CONV2D_MAX_K 15
+
+/*
+ * Single-channel 2D image filtering.
+ *   in   : H*W floats, row-major:        in[y*W + x]
+ *   filt : K*K floats, row-major:        filt[i*K + j]
+ *   out  : (H-K+1)*(W-K+1) floats, row-major, pitch W-K+1:
+ *          out[y*(W-K+1) + x] = sum_{i<K} sum_{j<K} in[(y+i)*W + x+j] * filt[i*K + j]
+ */
+int conv2d_single(const float *in, int H, int W, const float *filt, int K, float *out, void *stream);
+
+/*
+ * Multi-channel 2D convolution (Table I; layout DESIGN.md R13).
+ *   in   : N*C*H*W floats (NCHW)
+ *   filt : F*C*K*K floats (FCKK == torch OIHW)
+ *   out  : N*F*(H-K+1)*(W-K+1) floats (NFHoWo):
+ *          out[n][f][y][x] = sum_{c<C} sum_{i<K} sum_{j<K} in[n][c][y+i][x+j] * filt[f][c][i][j]
+ *   The filters of one F-block (all C channels) are staged in shared memory; F*C*K*K of any size
+ *   is supported (the F-block is sized to fit).
+ */
+int conv2d_multi(const float *in, int N, int C, int H, int W, const float *filt, int F, int K,
+                 float *out, void *stream);
+
+/*
+ * Same as conv2d_single / conv2d_multi with an explicit output-row band height per warp
+ * (band_h <= 0: the library's choice). For tuning sweeps and tests of the band / halo logic; the
+ * result is bitwise identical for every band_h (each output's summation order does not depend on
+ * its band).
+ */
+int conv2d_single_ex(const float *in, int H, int W, const float *filt, int K, float *out, void *stream,
+                     int band_h);
+int conv2d_multi_ex(const float *in, int N, int C, int H, int W, const float *filt, int F, int K,
+                    float *out, void *stream, int band_h);
+
+/*
+ * Baseline "direct convolution" of PAPER.md Fig. 1a: one thread per
+ * output element, each thread loads its K*K inputs itself (no column or row reuse). Same arguments,
+ * result and error codes as conv2d_single. Kept as the control for the memory-transaction evidence
+ * (profiles/); not a performance path.
+ */
+int conv2d_single_direct(const float *in, int H, int W, const float *filt, int K, float *out,
+                         void *stream);
+
+/* Human-readable text for a return code (static storage, never NULL). */
+const char *conv2d_strerror(int code);
+
+/* ABI version (major*100 + minor). */
+int conv2d_version(void);
+
+#ifdef __cplusplus
+}
+#endif
+
+#endif /* CONV2D_B200_H */

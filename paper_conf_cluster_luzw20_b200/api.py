@@ -1,0 +1,117 @@
+"""Tensor-level API over the C ABI (PyTorch supplies device memory and streams only).
+
+    out = conv2d_single(x, f)      # x: (H, W) fp32 CUDA, f: (K, K)      -> (H-K+1, W-K+1)
+    out = conv2d_multi(x, w)       # x: (N, C, H, W), w: (F, C, K, K)    -> (N, F, H-K+1, W-K+1)
+
+Every step of the computation runs in libconv2d.so's kernels; this module only checks types and
+shapes, allocates the output, and passes raw pointers plus the current stream. There is no CPU or
+eager-PyTorch fallback: non-CUDA tensors raise.
+
+`conv2d_single_host` / `conv2d_multi_host` are the end-to-end entry points for host-resident data:
+pinned host -> HBM copy, the kernel, HBM -> host copy, all on one stream (bench.py's `e2e`).
+"""
+from __future__ import annotations
+
+import torch
+
+from . import _capi
+
+
+def _stream_handle(stream) -> int:
+    s = stream if stream is not None else torch.cuda.current_stream()
+    return int(s.cuda_stream)
+
+
+def _check_dev(t: torch.Tensor, name: str):
+    if not isinstance(t, torch.Tensor):
+        raise TypeError(f"{name} must be a torch.Tensor")
+    if not t.is_cuda:
+        raise TypeError(f"{name} must be a CUDA tensor (no CPU fallback exists)")
+    if t.dtype != torch.float32:
+        raise TypeError(f"{name} must be float32, got {t.dtype}")
+    if not t.is_contiguous():
+        raise ValueError(f"{name} must be contiguous")
+
+
+def conv2d_single(x: torch.Tensor, f: torch.Tensor, out: torch.Tensor | None = None, stream=None,
+                  band_h: int = 0) -> torch.Tensor:
+    _check_dev(x, "x")
+    _check_dev(f, "f")
+    if x.dim() != 2 or f.dim() != 2 or f.shape[0] != f.shape[1]:
+        raise ValueError("x must be (H, W) and f (K, K)")
+    H, W = x.shape
+    K = f.shape[0]
+    if out is None:
+        out = torch.empty((max(H - K + 1, 0), max(W - K + 1, 0)), dtype=torch.float32, device=x.device)
+    else:
+        _check_dev(out, "out")
+        if tuple(out.shape) != (H - K + 1, W - K + 1):
+            raise ValueError("out has the wrong shape")
+    with torch.cuda.device(x.device):
+        _capi.check(_capi.conv2d_single_ex(x.data_ptr(), H, W, f.data_ptr(), K, out.data_ptr(),
+                                           _stream_handle(stream), band_h))
+    return out
+
+
+def conv2d_single_direct(x: torch.Tensor, f: torch.Tensor, out: torch.Tensor | None = None,
+                         stream=None) -> torch.Tensor:
+    """PAPER.md Fig. 1a baseline kernel (no column/row reuse); evidence control only."""
+    _check_dev(x, "x")
+    _check_dev(f, "f")
+    H, W = x.shape
+    K = f.shape[0]
+    if out is None:
+        out = torch.empty((H - K + 1, W - K + 1), dtype=torch.float32, device=x.device)
+    with torch.cuda.device(x.device):
+        _capi.check(_capi.conv2d_single_direct(x.data_ptr(), H, W, f.data_ptr(), K, out.data_ptr(),
+                                               _stream_handle(stream)))
+    return out
+
+
+def conv2d_multi(x: torch.Tensor, w: torch.Tensor, out: torch.Tensor | None = None, stream=None,
+                 band_h: int = 0) -> torch.Tensor:
+    _check_dev(x, "x")
+    _check_dev(w, "w")
+    if x.dim() != 4 or w.dim() != 4 or w.shape[1] != x.shape[1] or w.shape[2] != w.shape[3]:
+        raise ValueError("x must be (N, C, H, W) and w (F, C, K, K)")
+    N, C, H, W = x.shape
+    F, _, K, _ = w.shape
+    if out is None:
+        out = torch.empty((N, F, max(H - K + 1, 0), max(W - K + 1, 0)), dtype=torch.float32, device=x.device)
+    else:
+        _check_dev(out, "out")
+        if tuple(out.shape) != (N, F, H - K + 1, W - K + 1):
+            raise ValueError("out has the wrong shape")
+    with torch.cuda.device(x.device):
+        _capi.check(_capi.conv2d_multi_ex(x.data_ptr(), N, C, H, W, w.data_ptr(), F, K, out.data_ptr(),
+                                          _stream_handle(stream), band_h))
+    return out
+
+
+def conv2d_single_host(x_host: torch.Tensor, f_host: torch.Tensor, device="cuda", stream=None,
+                       out_host: torch.Tensor | None = None) -> torch.Tensor:
+    """End-to-end call on host tensors (pinned for async copies): H2D, kernel, D2H on one stream."""
+    dev = torch.device(device)
+    s = stream if stream is not None else torch.cuda.current_stream(dev)
+    with torch.cuda.stream(s):
+        x = x_host.to(dev, non_blocking=True)
+        f = f_host.to(dev, non_blocking=True)
+        y = conv2d_single(x, f, stream=s)
+        if out_host is None:
+            out_host = torch.empty(y.shape, dtype=torch.float32, pin_memory=True)
+        out_host.copy_(y, non_blocking=True)
+    return out_host
+
+
+def conv2d_multi_host(x_host: torch.Tensor, w_host: torch.Tensor, device="cuda", stream=None,
+                      out_host: torch.Tensor | None = None) -> torch.Tensor:
+    dev = torch.device(device)
+    s = stream if stream is not None else torch.cuda.current_stream(dev)
+    with torch.cuda.stream(s):
+        x = x_host.to(dev, non_blocking=True)
+        w = w_host.to(dev, non_blocking=True)
+        y = conv2d_multi(x, w, stream=s)
+        if out_host is None:
+            out_host = torch.empty(y.shape, dtype=torch.float32, pin_memory=True)
+        out_host.copy_(y, non_blocking=True)
+    return out_host

@@ -1,0 +1,470 @@
+// conv2d_kernels.cuh -- sm_100a kernels for direct, stride-1, valid-mode fp32 convolution with the
+// column reuse and row reuse of Lu, Zhang & Wang (Cluster 2020), re-designed for B200.
+//
+// Work decomposition:
+//   * One WARP owns a tile of 128*U output columns x BH output rows ("band"). Lane l holds the
+//     outputs x0 + 128u + 4l + {0..3} of every chunk u < U (V = 4 contiguous columns per lane, so
+//     every input-row load is one coalesced LDG.128 per lane and every output store is STG.128).
+//   * a1 Input row fetch: per input row, U LDG.128 per lane plus one extra LDG.128 on the first
+//     NE = ceil((K-1)/4) lanes (the K-1 halo columns right of the warp's span). Rows are prefetched
+//     PF rows ahead in registers.
+//   * a2 Column reuse (Sec. II-A, Alg. 1, Fig. 1c): the K-1 halo values
+//     a lane needs beyond its own 4 come from lanes l+1.. via __shfl_sync, never from memory. As in
+//     Alg. 1, the value a lane SUPPLIES is chosen with a static register index and a lane-dependent
+//     select (Alg. 1 lines 2-5 select by a 64-bit shift; here a SEL), so the window iTemp stays in
+//     registers. Halo element m (m = 4..K+2) of lane l lives in register
+//     m%4 of lane l + m/4: one SEL + one SHFL.IDX per (m, chunk), all indices compile-time.
+//   * a3 Row reuse (Sec. II-B, Alg. 2, flow P:303-311): each loaded input row is
+//     multiplied against all K filter rows into K output-row accumulators held in registers
+//     ("out ... can be stored in registers"). Slot q of the ring holds output row
+//     r-K+1+q after input row r; the update acc[q] = acc[q+1] + row . filter[K-1-q] SHIFTS the ring
+//     inside the first FMA of each chain, so the ring rotation costs no MOVs and every index is
+//     static (the dynamic->static index transformation of P:75-77). The first K-1 rows
+//     of a band (Alg. 2 case 1) skip the slots whose output row precedes the band; Alg. 2 case 3 is
+//     implicit (the band stops when its last output row completes).
+//   * a4 Filter supply: the CTA stages the filter into shared memory once (rows padded to KP floats)
+//     and the FMAs read it with broadcast LDS.128 (or from registers for K <= 5). Reentrant: no
+//     __constant__ state.
+//   * a5 Channel reduction (multi): for each input row, all C channels stream through the same
+//     accumulators; each thread also carries FB filters, so one window feeds FB*K*K*4 FMAs.
+//   * a6 Output store: slot 0 is complete after each row -> one coalesced store per lane; rows whose
+//     pitch breaks 16-byte alignment are realigned with warp shuffles (static per-shift variants).
+// Edge tiles (ragged right edge) and misaligned tensors take the same code with guarded scalar
+// loads/stores (SAFE=true).
+#pragma once
+
+#include <cstdint>
+#include <cuda_runtime.h>
+
+namespace c2d {
+
+constexpr unsigned kFull = 0xffffffffu;
+constexpr int kWarp = 32;
+constexpr int kCtaWarps = 4;  // 128 threads per CTA
+
+template <int K>
+struct KCfg {
+  static constexpr int NE = (K - 1 + 3) / 4;  // lanes that fetch the extra halo float4
+  static constexpr int KP = (K + 3) / 4 * 4;  // filter row padded to a multiple of 4 floats
+  static constexpr int WN = 4 + K - 1;        // window length per chunk: 4 outputs + K-1 halo
+};
+
+// ------------------------------------------------------------------------------------------------
+// memory helpers
+// ------------------------------------------------------------------------------------------------
+__device__ __forceinline__ float4 ldg4(const float *p) { return __ldg(reinterpret_cast<const float4 *>(p)); }
+
+__device__ __forceinline__ void stg4(float *p, float a, float b, float c, float d) {
+  __stcs(reinterpret_cast<float4 *>(p), make_float4(a, b, c, d));
+}
+
+// LDS.128 that the compiler may not hoist out of the row loop (keeps K*K filter values out of the
+// register file for large K).
+__device__ __forceinline__ void lds4_volatile(const float *p, float &a, float &b, float &c, float &d) {
+  const unsigned s = static_cast<unsigned>(__cvta_generic_to_shared(p));
+  asm volatile("ld.shared.v4.f32 {%0, %1, %2, %3}, [%4];" : "=f"(a), "=f"(b), "=f"(c), "=f"(d) : "r"(s));
+}
+
+// ------------------------------------------------------------------------------------------------
+// a1: one input row segment of a warp tile
+// ------------------------------------------------------------------------------------------------
+template <int K, int U>
+struct RowBuf {
+  float a[U][4];
+  float e[4];
+};
+
+// rowp points at input column 0 of the row. SAFE: guarded scalar loads (ragged edge / misaligned).
+template <int K, int U, bool SAFE>
+__device__ __forceinline__ void load_row(RowBuf<K, U> &b, const float *__restrict__ rowp, int x0, int W,
+                                         int lane) {
+#pragma unroll
+  for (int u = 0; u < U; ++u) {
+    const int x = x0 + 128 * u + 4 * lane;
+    if (!SAFE) {
+      const float4 v = ldg4(rowp + x);
+      b.a[u][0] = v.x; b.a[u][1] = v.y; b.a[u][2] = v.z; b.a[u][3] = v.w;
+    } else {
+#pragma unroll
+      for (int t = 0; t < 4; ++t) b.a[u][t] = (x + t < W) ? __ldg(rowp + x + t) : 0.f;
+    }
+  }
+#pragma unroll
+  for (int t = 0; t < 4; ++t) b.e[t] = 0.f;
+  if (KCfg<K>::NE > 0 && lane < KCfg<K>::NE) {
+    const int x = x0 + 128 * U + 4 * lane;
+    if (!SAFE && x + 3 < W) {
+      const float4 v = ldg4(rowp + x);
+      b.e[0] = v.x; b.e[1] = v.y; b.e[2] = v.z; b.e[3] = v.w;
+    } else {
+#pragma unroll
+      for (int t = 0; t < 4; ++t) b.e[t] = (x + t < W) ? __ldg(rowp + x + t) : 0.f;
+    }
+  }
+}
+
+// ------------------------------------------------------------------------------------------------
+// a2: column reuse -- assemble every chunk's window w[u][0..WN) = in[x0+128u+4l .. +WN)
+// ------------------------------------------------------------------------------------------------
+template <int K, int U>
+__device__ __forceinline__ void build_windows(const RowBuf<K, U> &b, float (&w)[U][KCfg<K>::WN], int lane) {
+#pragma unroll
+  for (int u = 0; u < U; ++u) {
+#pragma unroll
+    for (int t = 0; t < 4; ++t) w[u][t] = b.a[u][t];
+  }
+#pragma unroll
+  for (int m = 4; m < KCfg<K>::WN; ++m) {
+    const int d = m >> 2;  // source lane offset (static)
+    const int r = m & 3;   // source register (static)
+    const int src = (lane + d) & (kWarp - 1);
+#pragma unroll
+    for (int u = 0; u < U; ++u) {
+      // Lanes s < d supply the NEXT chunk's register r (for receivers that wrap past lane 31);
+      // lanes s >= d supply their own register r. Static register index, lane-dependent select.
+      const float nxt = (u + 1 < U) ? b.a[(u + 1 < U) ? u + 1 : 0][r] : b.e[r];
+      const float sup = (lane < d) ? nxt : b.a[u][r];
+      w[u][m] = __shfl_sync(kFull, sup, src);
+    }
+  }
+}
+
+// ------------------------------------------------------------------------------------------------
+// a4: filter row i as K registers
+// ------------------------------------------------------------------------------------------------
+template <int K, bool FREG>
+__device__ __forceinline__ void filter_row(float (&fr)[KCfg<K>::KP], const float *__restrict__ sf_row,
+                                           const float (&freg)[FREG ? K * K : 1], int i) {
+  if constexpr (FREG) {
+#pragma unroll
+    for (int j = 0; j < K; ++j) fr[j] = freg[i * K + j];
+  } else {
+#pragma unroll
+    for (int c = 0; c < KCfg<K>::KP / 4; ++c)
+      lds4_volatile(sf_row + 4 * c, fr[4 * c], fr[4 * c + 1], fr[4 * c + 2], fr[4 * c + 3]);
+  }
+}
+
+// ------------------------------------------------------------------------------------------------
+// a6: store 4 outputs per lane of a 128-wide output chunk starting at g (16B alignment unknown)
+// ------------------------------------------------------------------------------------------------
+template <int S>
+__device__ __forceinline__ void store_chunk_shifted(float *g, const float (&o)[4], int lane) {
+  // g is S floats past a 16-byte boundary. Lanes 0..30 store the aligned quad at g + 4 - S + 4l:
+  // own o[4-S..3] followed by lane l+1's o[0..3-S]. Lane 0 stores the 4-S head elements and lane 31
+  // the S tail elements with scalar stores.
+  float nb[4];
+#pragma unroll
+  for (int t = 0; t < 4; ++t) nb[t] = (t < 4 - S) ? __shfl_down_sync(kFull, o[t], 1) : 0.f;
+  float q[4];
+#pragma unroll
+  for (int k = 0; k < 4; ++k) q[k] = (k < S) ? o[(4 - S + k) & 3] : nb[(k - S) & 3];
+  if (lane < kWarp - 1) stg4(g + (4 - S) + 4 * lane, q[0], q[1], q[2], q[3]);
+  if (lane == 0) {
+#pragma unroll
+    for (int t = 0; t < 4 - S; ++t) __stcs(g + t, o[t]);
+  }
+  if (lane == kWarp - 1) {
+#pragma unroll
+    for (int t = 4 - S; t < 4; ++t) __stcs(g + 4 * (kWarp - 1) + t, o[t]);
+  }
+}
+
+__device__ __forceinline__ void store_chunk(float *g, const float (&o)[4], int lane) {
+  const int s = static_cast<int>((reinterpret_cast<uintptr_t>(g) >> 2) & 3);
+  switch (s) {  // warp-uniform: the dynamic shift becomes one of four static variants
+    case 0: stg4(g + 4 * lane, o[0], o[1], o[2], o[3]); break;
+    case 1: store_chunk_shifted<1>(g, o, lane); break;
+    case 2: store_chunk_shifted<2>(g, o, lane); break;
+    default: store_chunk_shifted<3>(g, o, lane); break;
+  }
+}
+
+template <int U, bool SAFE>
+__device__ __forceinline__ void store_row(float *__restrict__ orow, int x0, int Wo, const float (&o)[U][4],
+                                          int lane) {
+#pragma unroll
+  for (int u = 0; u < U; ++u) {
+    const int xb = x0 + 128 * u;
+    if (!SAFE) {
+      store_chunk(orow + xb, o[u], lane);
+    } else {
+#pragma unroll
+      for (int t = 0; t < 4; ++t) {
+        const int x = xb + 4 * lane + t;
+        if (x < Wo) __stcs(orow + x, o[u][t]);
+      }
+    }
+  }
+}
+
+// ------------------------------------------------------------------------------------------------
+// a3: row reuse -- one input row into the K-slot accumulator ring (single channel)
+// ------------------------------------------------------------------------------------------------
+template <int K, int U, bool FREG>
+__device__ __forceinline__ void row_reuse_single(float (&acc)[K][U][4], const float (&w)[U][KCfg<K>::WN],
+                                                 const float *__restrict__ sf,
+                                                 const float (&freg)[FREG ? K * K : 1], int qmin) {
+#pragma unroll
+  for (int q = 0; q < K; ++q) {
+    if (q >= qmin) {  // warp-uniform: the first K-1 rows of a band feed fewer outputs (Alg. 2 case 1)
+      const int i = K - 1 - q;  // filter row that input row r contributes to output row r-K+1+q
+      float fr[KCfg<K>::KP];
+      filter_row<K, FREG>(fr, sf + i * KCfg<K>::KP, freg, i);
+#pragma unroll
+      for (int u = 0; u < U; ++u) {
+#pragma unroll
+        for (int v = 0; v < 4; ++v) {
+          float s = (q + 1 < K) ? acc[(q + 1 < K) ? q + 1 : 0][u][v] : 0.f;  // ring shift
+#pragma unroll
+          for (int j = 0; j < K; ++j) s = fmaf(w[u][v + j], fr[j], s);
+          acc[q][u][v] = s;
+        }
+      }
+    }
+  }
+}
+
+// ------------------------------------------------------------------------------------------------
+// Single-channel kernel
+// ------------------------------------------------------------------------------------------------
+struct SingleArgs {
+  const float *in;
+  const float *filt;
+  float *out;
+  int H, W, Ho, Wo;
+  int band_h;     // output rows per warp tile
+  int n_cb;       // column blocks of 128*U outputs
+  int n_tiles;    // n_cb * n_bands
+  int aligned;    // in is 16B aligned and W % 4 == 0
+};
+
+template <int K, int U, int PF, bool SAFE>
+__device__ __forceinline__ void single_tile(const SingleArgs &a, const float *__restrict__ sf,
+                                            const float (&freg)[(K <= 5) ? K * K : 1], int x0, int ob, int oe,
+                                            int lane) {
+  constexpr bool FREG = (K <= 5);
+  const int rend = oe + K - 1;  // input rows [ob, rend)
+  const float *__restrict__ in = a.in;
+  RowBuf<K, U> buf[PF];
+#pragma unroll
+  for (int p = 0; p < PF; ++p)
+    if (ob + p < rend) load_row<K, U, SAFE>(buf[p], in + static_cast<size_t>(ob + p) * a.W, x0, a.W, lane);
+
+  float acc[K][U][4];
+#pragma unroll
+  for (int q = 0; q < K; ++q)
+#pragma unroll
+    for (int u = 0; u < U; ++u)
+#pragma unroll
+      for (int v = 0; v < 4; ++v) acc[q][u][v] = 0.f;
+
+  for (int r0 = ob; r0 < rend; r0 += PF) {
+#pragma unroll
+    for (int p = 0; p < PF; ++p) {
+      const int r = r0 + p;
+      if (r < rend) {
+        RowBuf<K, U> cur = buf[p];
+        if (r + PF < rend)
+          load_row<K, U, SAFE>(buf[p], in + static_cast<size_t>(r + PF) * a.W, x0, a.W, lane);
+        float w[U][KCfg<K>::WN];
+        build_windows<K, U>(cur, w, lane);
+        const int done = r - ob;  // rows of this band already streamed
+        const int qmin = (done < K - 1) ? (K - 1 - done) : 0;
+        row_reuse_single<K, U, FREG>(acc, w, sf, freg, qmin);
+        if (done >= K - 1) {  // slot 0 now holds the complete output row r-K+1
+          const float(&o)[U][4] = acc[0];
+          store_row<U, SAFE>(a.out + static_cast<size_t>(r - K + 1) * a.Wo, x0, a.Wo, o, lane);
+        }
+      }
+    }
+  }
+}
+
+template <int K, int U, int PF>
+__global__ void __launch_bounds__(kCtaWarps *kWarp) k_conv2d_single(const SingleArgs a) {
+  constexpr int KP = KCfg<K>::KP;
+  constexpr bool FREG = (K <= 5);
+  __shared__ __align__(16) float sf[K * KP];
+  for (int t = threadIdx.x; t < K * KP; t += blockDim.x) {
+    const int i = t / KP, j = t % KP;
+    sf[t] = (j < K) ? a.filt[i * K + j] : 0.f;
+  }
+  __syncthreads();
+  float freg[FREG ? K * K : 1];
+  if constexpr (FREG) {
+#pragma unroll
+    for (int i = 0; i < K; ++i)
+#pragma unroll
+      for (int j = 0; j < K; ++j) freg[i * K + j] = sf[i * KP + j];
+  } else {
+    freg[0] = 0.f;
+  }
+
+  const int lane = threadIdx.x & (kWarp - 1);
+  const int tile = blockIdx.x * kCtaWarps + (threadIdx.x >> 5);
+  if (tile >= a.n_tiles) return;
+  const int cb = tile % a.n_cb;
+  const int band = tile / a.n_cb;
+  const int x0 = cb * 128 * U;
+  const int ob = band * a.band_h;
+  const int oe = min(ob + a.band_h, a.Ho);
+  const bool fast = a.aligned && (x0 + 128 * U <= a.Wo);  // warp-uniform
+  if (fast)
+    single_tile<K, U, PF, false>(a, sf, freg, x0, ob, oe, lane);
+  else
+    single_tile<K, U, PF, true>(a, sf, freg, x0, ob, oe, lane);
+}
+
+// ------------------------------------------------------------------------------------------------
+// Multi-channel kernel: FB filters per warp, C channels streamed per input row
+// ------------------------------------------------------------------------------------------------
+struct MultiArgs {
+  const float *in;
+  const float *filt;
+  float *out;
+  int N, C, H, W, F, Ho, Wo;
+  int band_h, n_cb, n_bands, n_fb;
+  long long n_tiles;
+  int aligned;
+};
+
+// sfc: staged filters of channel c, layout [K][FB][KP] (filter row i of filter fb at (i*FB+fb)*KP)
+template <int K, int FB, bool SHIFT>
+__device__ __forceinline__ void row_reuse_multi(float (&acc)[K][FB][4], const float (&w)[KCfg<K>::WN],
+                                                const float *__restrict__ sfc, int qmin) {
+  constexpr int KP = KCfg<K>::KP;
+#pragma unroll
+  for (int q = 0; q < K; ++q) {
+    if (q >= qmin) {
+      const int i = K - 1 - q;
+#pragma unroll
+      for (int fb = 0; fb < FB; ++fb) {
+        float fr[KP];
+#pragma unroll
+        for (int c4 = 0; c4 < KP / 4; ++c4)
+          lds4_volatile(sfc + (i * FB + fb) * KP + 4 * c4, fr[4 * c4], fr[4 * c4 + 1], fr[4 * c4 + 2],
+                        fr[4 * c4 + 3]);
+#pragma unroll
+        for (int v = 0; v < 4; ++v) {
+          float s;
+          if (SHIFT)
+            s = (q + 1 < K) ? acc[(q + 1 < K) ? q + 1 : 0][fb][v] : 0.f;
+          else
+            s = acc[q][fb][v];
+#pragma unroll
+          for (int j = 0; j < K; ++j) s = fmaf(w[v + j], fr[j], s);
+          acc[q][fb][v] = s;
+        }
+      }
+    }
+  }
+}
+
+template <int K, int FB, bool SAFE>
+__device__ __forceinline__ void multi_tile(const MultiArgs &a, const float *__restrict__ sf, int n, int f0,
+                                           int x0, int ob, int oe, int lane) {
+  constexpr int KP = KCfg<K>::KP;
+  const int rend = oe + K - 1;
+  const int C = a.C;
+  const size_t plane = static_cast<size_t>(a.H) * a.W;
+  const float *__restrict__ img = a.in + static_cast<size_t>(n) * C * plane;
+
+  float acc[K][FB][4];
+#pragma unroll
+  for (int q = 0; q < K; ++q)
+#pragma unroll
+    for (int fb = 0; fb < FB; ++fb)
+#pragma unroll
+      for (int v = 0; v < 4; ++v) acc[q][fb][v] = 0.f;
+
+  RowBuf<K, 1> nxt;
+  load_row<K, 1, SAFE>(nxt, img + static_cast<size_t>(ob) * a.W, x0, a.W, lane);
+  for (int r = ob; r < rend; ++r) {
+    const int done = r - ob;
+    const int qmin = (done < K - 1) ? (K - 1 - done) : 0;
+    for (int c = 0; c < C; ++c) {
+      RowBuf<K, 1> cur = nxt;
+      // prefetch the next (row, channel) of the stream
+      {
+        int rn = r, cn = c + 1;
+        if (cn == C) { cn = 0; ++rn; }
+        if (rn < rend)
+          load_row<K, 1, SAFE>(nxt, img + cn * plane + static_cast<size_t>(rn) * a.W, x0, a.W, lane);
+      }
+      float w[1][KCfg<K>::WN];
+      build_windows<K, 1>(cur, w, lane);
+      const float *sfc = sf + static_cast<size_t>(c) * K * FB * KP;
+      if (c == 0)
+        row_reuse_multi<K, FB, true>(acc, w[0], sfc, qmin);
+      else
+        row_reuse_multi<K, FB, false>(acc, w[0], sfc, qmin);
+    }
+    if (done >= K - 1) {
+      const int o = r - K + 1;
+#pragma unroll
+      for (int fb = 0; fb < FB; ++fb) {
+        if (f0 + fb < a.F) {
+          float *orow = a.out + ((static_cast<size_t>(n) * a.F + f0 + fb) * a.Ho + o) * a.Wo;
+          const float(&ov)[1][4] = *reinterpret_cast<const float(*)[1][4]>(&acc[0][fb][0]);
+          store_row<1, SAFE>(orow, x0, a.Wo, ov, lane);
+        }
+      }
+    }
+  }
+}
+
+template <int K, int FB>
+__global__ void __launch_bounds__(kCtaWarps *kWarp) k_conv2d_multi(const MultiArgs a) {
+  constexpr int KP = KCfg<K>::KP;
+  extern __shared__ __align__(16) float smem[];
+  // CTA = 4 warps on the same (n, F-block): stage that block's filters, layout [C][K][FB][KP]
+  const long long cta_tile0 = static_cast<long long>(blockIdx.x) * kCtaWarps;
+  const long long per_fb = static_cast<long long>(a.n_cb) * a.n_bands;  // tiles per (n, F-block)
+  const int fblk = static_cast<int>((cta_tile0 / per_fb) % a.n_fb);
+  // host guarantees per_fb % kCtaWarps == 0, so all warps of the CTA share (n, fblk)
+  const int f0 = fblk * FB;
+  const int C = a.C;
+  const int total = C * K * FB * KP;
+  for (int t = threadIdx.x; t < total; t += blockDim.x) {
+    const int j = t % KP;
+    const int fb = (t / KP) % FB;
+    const int i = (t / (KP * FB)) % K;
+    const int c = t / (KP * FB * K);
+    const int f = f0 + fb;
+    smem[t] = (j < K && f < a.F) ? a.filt[((static_cast<size_t>(f) * C + c) * K + i) * K + j] : 0.f;
+  }
+  __syncthreads();
+
+  const int lane = threadIdx.x & (kWarp - 1);
+  const long long tile = cta_tile0 + (threadIdx.x >> 5);
+  if (tile >= a.n_tiles) return;
+  const int cb = static_cast<int>(tile % a.n_cb);
+  const int band = static_cast<int>((tile / a.n_cb) % a.n_bands);
+  const int n = static_cast<int>(tile / (per_fb * a.n_fb));
+  const int x0 = cb * 128;
+  const int ob = band * a.band_h;
+  const int oe = min(ob + a.band_h, a.Ho);
+  if (ob >= a.Ho) return;
+  const bool fast = a.aligned && (x0 + 128 <= a.Wo);
+  if (fast)
+    multi_tile<K, FB, false>(a, smem, n, f0, x0, ob, oe, lane);
+  else
+    multi_tile<K, FB, true>(a, smem, n, f0, x0, ob, oe, lane);
+}
+
+// ------------------------------------------------------------------------------------------------
+// Baseline: PAPER.md Fig. 1a direct convolution, one thread per output, K*K loads per thread
+// ------------------------------------------------------------------------------------------------
+__global__ void __launch_bounds__(256) k_conv2d_direct(const float *__restrict__ in, int W, const float *__restrict__ filt,
+                                                       int K, float *__restrict__ out, int Ho, int Wo) {
+  const long long idx = static_cast<long long>(blockIdx.x) * blockDim.x + threadIdx.x;
+  if (idx >= static_cast<long long>(Ho) * Wo) return;
+  const int y = static_cast<int>(idx / Wo), x = static_cast<int>(idx % Wo);
+  float s = 0.f;
+  for (int i = 0; i < K; ++i)
+    for (int j = 0; j < K; ++j) s = fmaf(in[static_cast<size_t>(y + i) * W + x + j], __ldg(filt + i * K + j), s);
+  out[idx] = s;
+}
+
+}  // namespace c2d

@@ -1,0 +1,103 @@
+"""CPU-side checks of the boundary: libconv2d.so builds for sm_100a, loads, and exports every symbol
+include/conv2d.h declares; the binding mirrors the header; host-side argument errors are reported
+without touching a GPU. No compute calls (no GPU here)."""
+import ctypes
+import os
+import re
+import subprocess
+
+import pytest
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+HEADER = os.path.join(ROOT, "include", "conv2d.h")
+
+
+@pytest.fixture(scope="module")
+def lib():
+    from paper_conf_cluster_luzw20_b200 import _build, _capi
+
+    _build.build()
+    return _capi.load()
+
+
+def _declared_functions():
+    text = open(HEADER).read()
+    text = re.sub(r"/\*.*?\*/", "", text, flags=re.S)
+    return sorted(set(re.findall(r"^\s*(?:const\s+)?\w+\s*\*?\s*(conv2d_\w+)\s*\(", text, flags=re.M)))
+
+
+def test_header_declares_the_boundary():
+    funcs = _declared_functions()
+    for f in ("conv2d_single", "conv2d_multi", "conv2d_strerror"):
+        assert f in funcs
+
+
+def test_every_declared_symbol_is_exported(lib):
+    from paper_conf_cluster_luzw20_b200 import _capi
+
+    funcs = _declared_functions()
+    assert sorted(funcs) == sorted(_capi.EXPORTS)
+    for f in funcs:
+        assert hasattr(lib, f), f
+    out = subprocess.run(["nm", "-D", "--defined-only", _capi.LIB_PATH], capture_output=True, text=True).stdout
+    for f in funcs:
+        assert re.search(rf"\bT {f}$", out, flags=re.M), f"{f} not exported with C linkage"
+
+
+def test_error_codes_match_header(lib):
+    from paper_conf_cluster_luzw20_b200 import _capi
+
+    text = open(HEADER).read()
+    codes = {m[0]: int(m[1]) for m in re.findall(r"#define (CONV2D_\w+) \(?(-?\d+)\)?", text)}
+    assert codes["CONV2D_OK"] == _capi.CONV2D_OK
+    assert codes["CONV2D_ENULL"] == _capi.CONV2D_ENULL
+    assert codes["CONV2D_ESHAPE"] == _capi.CONV2D_ESHAPE
+    assert codes["CONV2D_EK"] == _capi.CONV2D_EK
+    assert codes["CONV2D_EOVERLAP"] == _capi.CONV2D_EOVERLAP
+    assert codes["CONV2D_ECUDA"] == _capi.CONV2D_ECUDA
+    assert codes["CONV2D_EALIGN"] == _capi.CONV2D_EALIGN
+    assert codes["CONV2D_MAX_K"] == _capi.CONV2D_MAX_K
+    for c in codes.values():
+        assert isinstance(_capi.strerror(c), str) and _capi.strerror(c)
+    assert lib.conv2d_version() >= 100
+
+
+def test_argument_errors_need_no_gpu(lib):
+    """Validation happens before any CUDA call: these return their codes on a GPU-less host."""
+    from paper_conf_cluster_luzw20_b200 import _capi as c
+
+    a, b, o = 0x10000, 0x20000000, 0x40000000  # fake, never dereferenced
+    assert c.conv2d_single(None, 8, 8, b, 3, o) == c.CONV2D_ENULL
+    assert c.conv2d_single(a, 8, 8, None, 3, o) == c.CONV2D_ENULL
+    assert c.conv2d_single(a, 8, 8, b, 16, o) == c.CONV2D_EK
+    assert c.conv2d_single(a, 8, 8, b, 0, o) == c.CONV2D_ESHAPE
+    assert c.conv2d_single(a, 2, 8, b, 3, o) == c.CONV2D_ESHAPE
+    assert c.conv2d_single(a, 8, 2, b, 3, o) == c.CONV2D_ESHAPE
+    assert c.conv2d_single(a + 2, 8, 8, b, 3, o) == c.CONV2D_EALIGN
+    assert c.conv2d_single(a, 8, 8, b, 3, a + 16) == c.CONV2D_EOVERLAP
+    assert c.conv2d_single(a, 8, 8, b, 3, b) == c.CONV2D_EOVERLAP
+    assert c.conv2d_multi(a, 0, 1, 8, 8, b, 1, 3, o) == c.CONV2D_ESHAPE
+    assert c.conv2d_multi(a, 1, 0, 8, 8, b, 1, 3, o) == c.CONV2D_ESHAPE
+    assert c.conv2d_multi(a, 1, 1, 8, 8, b, 0, 3, o) == c.CONV2D_ESHAPE
+    assert c.conv2d_multi(a, 1, 1, 8, 8, b, 1, 16, o) == c.CONV2D_EK
+    assert c.conv2d_multi(a, 2, 2, 8, 8, b, 1, 3, a + 100) == c.CONV2D_EOVERLAP
+    assert c.conv2d_single_direct(a, 8, 8, b, 20, o) == c.CONV2D_EK
+
+
+def test_library_is_sm100a(lib):
+    from paper_conf_cluster_luzw20_b200 import _capi
+
+    out = subprocess.run(["/usr/local/cuda/bin/cuobjdump", "--list-elf", _capi.LIB_PATH],
+                         capture_output=True, text=True).stdout
+    assert "sm_100a" in out
+
+
+def test_product_path_has_no_oracle_dependency():
+    """The package never imports or links the oracle (they share no code)."""
+    pkg = os.path.join(ROOT, "paper_conf_cluster_luzw20_b200")
+    for dirpath, _, files in os.walk(pkg):
+        for fn in files:
+            if fn.endswith((".py", ".cu", ".cuh", ".h", ".c", ".cpp")):
+                src = open(os.path.join(dirpath, fn)).read()
+                assert "import oracle" not in src and "from oracle" not in src, fn
+                assert "liboracle" not in src and "conv2d_oracle" not in src, fn

@@ -1,0 +1,95 @@
+"""GPU parity of conv2d_multi (C ABI via the binding) against the CPU oracle: small shapes element by
+element for every K, F not a multiple of the F-block, ragged widths; the BASELINE.json multi-channel
+configs at full size on sampled outputs (plus full images for a subset of the batch)."""
+import numpy as np
+import pytest
+import torch
+
+import paper_conf_cluster_luzw20_b200 as pkg
+from gen import synth
+from tests.gpu_helpers import check_full_multi, check_full_single, check_points_multi, dev_image
+
+pytestmark = pytest.mark.gpu
+DEV = "cuda"
+
+
+def _w(F, C, K, dist="he", seed=5):
+    return torch.from_numpy(synth.make_filter(seed, K, dist, F=F, C=C)).to(DEV)
+
+
+@pytest.mark.parametrize("K", list(range(1, 16)))
+def test_all_k_small(cuda_device, K):
+    for (N, C, F, dh, dw) in [(1, 1, 1, 0, 0), (2, 3, 5, 7, 40), (1, 2, 9, 3, 131), (3, 1, 3, 20, 9)]:
+        x = dev_image((N, C, K + dh, K + dw), "sym", seed=K + N)
+        w = _w(F, C, K, seed=K)
+        check_full_multi(x, w, pkg.conv2d_multi(x, w))
+
+
+@pytest.mark.parametrize("K", [1, 3, 5, 7, 15])
+def test_integer_bitwise(cuda_device, K):
+    x = dev_image((2, 3, K + 17, 260), "int", seed=K)
+    w = _w(7, 3, K, "int", seed=K)
+    check_full_multi(x, w, pkg.conv2d_multi(x, w), exact=True)
+
+
+def test_reduces_to_single(cuda_device):
+    for K in (3, 7):
+        x = dev_image((1, 1, 90, 300), "img", seed=K)
+        w = _w(1, 1, K, "rand")
+        ym = pkg.conv2d_multi(x, w)
+        ys = pkg.conv2d_single(x[0, 0].contiguous(), w[0, 0].contiguous())
+        check_full_single(x[0, 0], w[0, 0], ys)
+        check_full_multi(x, w, ym)
+
+
+def test_band_and_batch_split_bitwise(cuda_device):
+    """Band height and batch sharding leave every output bit unchanged."""
+    x = dev_image((6, 3, 70, 150), "img")
+    w = _w(10, 3, 5)
+    ref = pkg.conv2d_multi(x, w)
+    for bh in (1, 3, 11, 1000):
+        assert torch.equal(pkg.conv2d_multi(x, w, band_h=bh), ref)
+    assert torch.equal(pkg.conv2d_multi(x[2:5].contiguous(), w), ref[2:5])
+    assert torch.equal(pkg.conv2d_multi(x, w[3:8].contiguous()), ref[:, 3:8])
+
+
+def test_config2_resnet_3x3(cuda_device):
+    """configs[2]: N=32, C=F=64, 56x56, K=3 -- images 0 and 31 in full, sampled points elsewhere."""
+    N, C, F, S, K = 32, 64, 64, 56, 3
+    x = dev_image((N, C, S, S), "sym", seed=synth.BASE_SEED + 2)
+    w = _w(F, C, K, "he", seed=synth.BASE_SEED + 2)
+    y = pkg.conv2d_multi(x, w)
+    check_full_multi(x[[0, N - 1]].contiguous(), w, y[[0, N - 1]].contiguous())
+    rng = np.random.default_rng(2)
+    P = 600
+    check_points_multi(x, w, y, rng.integers(0, N, P), rng.integers(0, F, P), rng.integers(0, S - K + 1, P),
+                       rng.integers(0, S - K + 1, P))
+
+
+def test_config3_small_c_large_k(cuda_device):
+    """configs[3]: N=128, C=3, F=64, 224x224, K=7 (R16: N=128) -- sampled + image 5 full."""
+    N, C, F, S, K = 128, 3, 64, 224, 7
+    x = dev_image((N, C, S, S), "img", seed=synth.BASE_SEED + 3)
+    w = _w(F, C, K, "he", seed=synth.BASE_SEED + 3)
+    y = pkg.conv2d_multi(x, w)
+    torch.cuda.synchronize()
+    check_full_multi(x[5:6].contiguous(), w[:9].contiguous(), y[5:6, :9].contiguous())
+    rng = np.random.default_rng(3)
+    P = 800
+    Ho = S - K + 1
+    ns = np.concatenate([rng.integers(0, N, P), [0, N - 1, N - 1, 0]])
+    fs = np.concatenate([rng.integers(0, F, P), [0, F - 1, 0, F - 1]])
+    ys = np.concatenate([rng.integers(0, Ho, P), [0, Ho - 1, Ho - 1, 0]])
+    xs = np.concatenate([rng.integers(0, Ho, P), [Ho - 1, 0, Ho - 1, 0]])
+    check_points_multi(x, w, y, ns, fs, ys, xs)
+
+
+@pytest.mark.parametrize("layer", [("CONV1", 28, 128, 3), ("CONV3", 12, 64, 5), ("CONV4", 14, 16, 5),
+                                   ("CONV10", 112, 128, 3)])
+def test_table1_layers(cuda_device, layer):
+    """PAPER.md Table I layer shapes at C in {1, 3}, reduced batch, every output."""
+    name, S, F, K = layer
+    for C in (1, 3):
+        x = dev_image((4, C, S, S), "img", seed=S + C)
+        w = _w(F, C, K, "he", seed=F)
+        check_full_multi(x, w, pkg.conv2d_multi(x, w))

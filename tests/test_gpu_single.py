@@ -1,0 +1,168 @@
+"""GPU parity of conv2d_single (C ABI via the binding) against the CPU oracle.
+
+Small shapes are compared element by element (all K in 1..15, ragged widths, every W % 4, Wo < 32,
+H == K, W == K, misaligned pointers); the BASELINE.json configs at full size are compared on sampled
+outputs (corners, edges, band boundaries, random points) in the launch configuration bench.py times.
+"""
+import numpy as np
+import pytest
+import torch
+
+import paper_conf_cluster_luzw20_b200 as pkg
+from gen import synth
+from paper_conf_cluster_luzw20_b200 import _capi
+from tests.gpu_helpers import (check_full_single, check_points_single, dev_image, sample_points)
+
+pytestmark = pytest.mark.gpu
+DEV = "cuda"
+
+
+def _filt(K, dist="rand", seed=3):
+    return torch.from_numpy(synth.make_filter(seed, K, dist)[0, 0]).to(DEV)
+
+
+def test_config0_256_k3(cuda_device):
+    """BASELINE.json configs[0]: 256x256, 3x3, valid, stride 1 -- every output."""
+    x = dev_image((256, 256), "img")
+    for dist in ("rand", "gauss", "box"):
+        f = _filt(3, dist)
+        check_full_single(x, f, pkg.conv2d_single(x, f))
+
+
+SMALL_SHAPES = [(0, 0), (1, 3), (9, 4), (37, 300), (70, 517), (33, 1023), (20, 1030), (150, 256)]
+
+
+@pytest.mark.parametrize("K", list(range(1, 16)))
+def test_all_k_small_shapes(cuda_device, K):
+    rng = np.random.default_rng(K)
+    for (dh, dw) in SMALL_SHAPES:
+        H, W = K + dh, K + dw
+        x = dev_image((H, W), "sym", seed=K * 1000 + dh)
+        f = _filt(K, "rand", seed=K)
+        check_full_single(x, f, pkg.conv2d_single(x, f))
+    # one random non-trivial band height on a taller image: several bands and a ragged last band
+    x = dev_image((K + 75, 389), "img", seed=K)
+    f = _filt(K, "gauss")
+    check_full_single(x, f, pkg.conv2d_single(x, f, band_h=int(rng.integers(1, 20))))
+
+
+@pytest.mark.parametrize("K", [1, 2, 3, 4, 5, 7, 9, 11, 13, 15])
+def test_integer_data_bitwise(cuda_device, K):
+    """Integer data: every fp32 partial sum is exact, so the GPU must equal the oracle bit for bit."""
+    for (H, W) in [(K + 40, 517), (K + 3, 1024), (2 * K + 1, 131)]:
+        x = dev_image((H, W), "int", seed=H + K)
+        f = _filt(K, "int", seed=K)
+        check_full_single(x, f, pkg.conv2d_single(x, f), exact=True)
+
+
+@pytest.mark.parametrize("K", [3, 5, 8, 15])
+def test_misaligned_pointers(cuda_device, K):
+    """in / out offset by 1..3 floats from 16-byte alignment take the scalar / shifted-store paths."""
+    H, W = K + 50, 600
+    for off_in in (0, 1, 2, 3):
+        for off_out in (0, 1, 3):
+            xb = dev_image((H * W + 4,), "img", seed=off_in)
+            x = xb[off_in:off_in + H * W].view(H, W)
+            ob = torch.empty((H - K + 1) * (W - K + 1) + 4, device=DEV)
+            y = ob[off_out:off_out + (H - K + 1) * (W - K + 1)].view(H - K + 1, W - K + 1)
+            f = _filt(K)
+            pkg.conv2d_single(x, f, out=y)
+            check_full_single(x, f, y)
+
+
+@pytest.mark.parametrize("K", [1, 3, 6, 15])
+def test_band_height_does_not_change_bits(cuda_device, K):
+    """Every output's summation order is independent of its band (and so of any row-band shard)."""
+    x = dev_image((K + 300, 700), "img", seed=K)
+    f = _filt(K)
+    ref = pkg.conv2d_single(x, f)
+    for bh in (1, 2, 5, 17, 64, 10 ** 6):
+        assert torch.equal(pkg.conv2d_single(x, f, band_h=bh), ref)
+    # a row sub-range computed on its own (what a row-band shard does) equals the matching rows
+    r0, r1 = 37, 201
+    sub = pkg.conv2d_single(x[r0:r1 + K - 1].contiguous(), f)
+    assert torch.equal(sub, ref[r0:r1])
+
+
+def test_nan_receptive_field(cuda_device):
+    K, H, W = 5, 80, 300
+    x = dev_image((H, W), "img")
+    r, c = 41, 133
+    x[r, c] = float("nan")
+    y = pkg.conv2d_single(x, _filt(K)).cpu().numpy()
+    mask = np.zeros(y.shape, bool)
+    mask[r - K + 1:r + 1, c - K + 1:c + 1] = True
+    assert np.array_equal(np.isnan(y), mask)
+
+
+def test_closed_forms_on_gpu(cuda_device):
+    x = dev_image((200, 333), "img")
+    for K in (3, 7, 15):
+        d = torch.zeros((K, K), device=DEV)
+        d[K // 2, K - 1] = 1.0
+        y = pkg.conv2d_single(x, d)
+        assert torch.equal(y, x[K // 2:K // 2 + 200 - K + 1, K - 1:K - 1 + 333 - K + 1])
+    c = torch.full((64, 300), 0.75, device=DEV)
+    f = _filt(9, "int")
+    assert (pkg.conv2d_single(c, f) == 0.75 * float(f.double().sum())).all()
+
+
+def test_direct_baseline_kernel(cuda_device):
+    for K in (3, 5, 15):
+        x = dev_image((K + 60, 257), "img", seed=K)
+        f = _filt(K)
+        check_full_single(x, f, pkg.conv2d_single_direct(x, f))
+
+
+def test_error_codes_on_device(cuda_device):
+    x = torch.zeros((10, 10), device=DEV)
+    f = torch.zeros((3, 3), device=DEV)
+    y = torch.zeros((8, 8), device=DEV)
+    assert _capi.conv2d_single(x.data_ptr(), 10, 10, f.data_ptr(), 16, y.data_ptr()) == _capi.CONV2D_EK
+    assert _capi.conv2d_single(x.data_ptr(), 10, 10, f.data_ptr(), 3, x.data_ptr() + 8) == _capi.CONV2D_EOVERLAP
+    with pytest.raises(TypeError):
+        pkg.conv2d_single(x.cpu(), f.cpu())  # no CPU fallback
+    with pytest.raises(_capi.Conv2dError):
+        pkg.conv2d_single(torch.zeros((2, 10), device=DEV), f)
+
+
+# --------------------------------------------------------------------------------------------
+# BASELINE.json configs at full size, sampled outputs
+# --------------------------------------------------------------------------------------------
+@pytest.mark.parametrize("S", [1024, 2048, 4096, 8192])
+def test_config1_sweep_full_size_sampled(cuda_device, S):
+    """configs[1]: 1024^2..8192^2 x K in {3,..,15}, the bench launch configuration, sampled."""
+    rng = np.random.default_rng(S)
+    x = dev_image((S, S), "img", seed=synth.BASE_SEED + 1)
+    for K in (3, 5, 7, 9, 11, 13, 15):
+        f = _filt(K, "rand", seed=synth.BASE_SEED + K)
+        y = pkg.conv2d_single(x, f)
+        torch.cuda.synchronize()
+        ys, xs = sample_points(S - K + 1, S - K + 1, 400, rng, band_h=None)
+        check_points_single(x, f, y, ys, xs)
+        assert torch.isfinite(y).all()
+    del x, y
+
+
+def test_config4_32768_k15_sampled(cuda_device):
+    """configs[4]: one 32768^2 image, K=15 (4 GiB in + 4 GiB out) on one B200, sampled; and the
+    row-band split used across GPUs reproduces it bit for bit at the band seams."""
+    S, K = 32768, 15
+    free, _ = torch.cuda.mem_get_info()
+    if free < 10 * (1 << 30):
+        pytest.skip("needs ~9 GiB of free HBM")
+    x = dev_image((S, S), "img", seed=synth.BASE_SEED + 4)
+    f = _filt(K, "gauss")
+    y = pkg.conv2d_single(x, f)
+    torch.cuda.synchronize()
+    rng = np.random.default_rng(4)
+    Ho = S - K + 1
+    ys, xs = sample_points(Ho, Ho, 300, rng)
+    check_points_single(x, f, y, ys, xs)
+    # 8 row bands computed independently (the multi-GPU decomposition) match at the seams
+    bands = np.linspace(0, Ho, 9).astype(int)
+    for b in range(8):
+        o0, o1 = int(bands[b]), int(bands[b + 1])
+        lo, hi = max(o0, o1 - 3), o1
+        part = pkg.conv2d_single(x[lo:hi + K - 1], f)
+        assert torch.equal(part, y[lo:hi])
