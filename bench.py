@@ -1,0 +1,542 @@
+#!/usr/bin/env python
+"""Benchmark of the hot path (driver contract).
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference] [--workload NAME]
+
+Default workload = BASELINE.json configs[1], the workload its metric is quoted on: the single-channel
+sweep of 1024^2, 2048^2, 4096^2, 8192^2 fp32 images x K in {3,5,7,9,11,13,15} (28 convolutions).
+One "step" = one pass of the whole hot path over that sweep: every (size, K) point is one
+conv2d_single call on its own input/output buffers (so no point reads another's data from L2),
+largest images first. `value` = output pixels of all points of all ranks / time (Gpixel/s), timed on
+the device with CUDA events, L2 flushed (a 512 MiB write) between steps outside the timed region.
+
+N > 1 (torchrun): every rank runs the same sweep on its own images (seeded by rank): weak scaling,
+no data-path collective (north_star: "partitioned ... by image/batch ... no collective needed").
+Other workloads (--workload): config0, config2, config3 (GFLOP/s), config4 (32768^2 K=15; at N>1
+row bands with the NCCL halo exchange of shard.py).
+
+--impl reference: the CPU oracle (this tier's reference arm) timed as it stands on the host cores,
+on a bounded sample of the same workload (rank 0 only).
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import math
+import os
+import statistics
+import sys
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+if ROOT not in sys.path:
+    sys.path.insert(0, ROOT)
+
+BASELINE_METRIC = "conv2d Gpixel/s and multi-channel GFLOP/s (fp32) at 1/2/4/8 B200, % roofline"
+SWEEP_SIZES = (8192, 4096, 2048, 1024)
+SWEEP_KS = (3, 5, 7, 9, 11, 13, 15)
+N_SM = 148
+FMA_LANES_PER_SM = 128
+
+
+def load_peaks():
+    p = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    try:
+        with open(p) as fh:
+            d = json.load(fh)
+        return {"hbm_gbs": float(d["hbm_gbs"]), "sm_max_mhz": float(d.get("sm_max_mhz", 1965.0)),
+                "source": "measured (MEASURED_PEAKS.json)"}
+    except Exception:
+        return {"hbm_gbs": 6650.0, "sm_max_mhz": 1965.0, "source": "fallback (B200_PROFILING.md)"}
+
+
+def fp32_fma_peak_tflops(sm_mhz):
+    """fp32 CUDA-core peak: 148 SMs x 128 FMA lanes x 2 flop x clock."""
+    return N_SM * FMA_LANES_PER_SM * 2 * sm_mhz * 1e6 / 1e12
+
+
+# ------------------------------------------------------------------------------------------------
+# workloads
+# ------------------------------------------------------------------------------------------------
+class Point:
+    """One conv call of a step: shapes, device buffers, algorithmic work."""
+
+    def __init__(self, kind, name, dims, K):
+        self.kind, self.name, self.dims, self.K = kind, name, dims, K
+        self.x = self.f = self.y = None
+
+    @property
+    def out_px(self):
+        if self.kind == "single":
+            H, W = self.dims
+            return (H - self.K + 1) * (W - self.K + 1)
+        N, C, H, W, F = self.dims
+        return N * F * (H - self.K + 1) * (W - self.K + 1)
+
+    @property
+    def flops(self):
+        C = 1 if self.kind == "single" else self.dims[1]
+        return 2.0 * self.out_px * C * self.K * self.K
+
+    @property
+    def bytes(self):
+        """compulsory HBM bytes: inputs + outputs + filters"""
+        if self.kind == "single":
+            H, W = self.dims
+            return 4.0 * (H * W + self.out_px + self.K * self.K)
+        N, C, H, W, F = self.dims
+        return 4.0 * (N * C * H * W + self.out_px + F * C * self.K * self.K)
+
+    def in_bytes(self):
+        if self.kind == "single":
+            return 4 * self.dims[0] * self.dims[1]
+        N, C, H, W, F = self.dims
+        return 4 * N * C * H * W
+
+    def filt_bytes(self):
+        C = 1 if self.kind == "single" else self.dims[1]
+        F = 1 if self.kind == "single" else self.dims[4]
+        return 4 * F * C * self.K * self.K
+
+    def bound(self, peaks, sm_mhz):
+        t_mem = self.bytes / (peaks["hbm_gbs"] * 1e9)
+        t_fma = self.flops / (fp32_fma_peak_tflops(sm_mhz) * 1e12)
+        return ("hbm", t_mem) if t_mem >= t_fma else ("alu", t_fma)
+
+
+def workload_points(name):
+    if name == "sweep":
+        return [Point("single", f"{S}^2 K={K}", (S, S), K) for S in SWEEP_SIZES for K in SWEEP_KS], \
+            "Gpixel/s"
+    if name == "config0":
+        return [Point("single", "256^2 K=3", (256, 256), 3)], "Gpixel/s"
+    if name == "config2":
+        return [Point("multi", "N32 C64 F64 56^2 K3", (32, 64, 56, 56, 64), 3)], "GFLOP/s"
+    if name == "config3":
+        return [Point("multi", "N128 C3 F64 224^2 K7", (128, 3, 224, 224, 64), 7)], "GFLOP/s"
+    if name == "config4":
+        return [Point("single", "32768^2 K=15", (32768, 32768), 15)], "Gpixel/s"
+    raise SystemExit(f"unknown workload {name}")
+
+
+WORKLOAD_DESC = {
+    "sweep": "BASELINE.json configs[1]: single-channel sweep, 1024^2/2048^2/4096^2/8192^2 x K in "
+             "{3,5,7,9,11,13,15} (28 conv2d_single calls per step, largest first)",
+    "config0": "BASELINE.json configs[0]: 256x256, K=3",
+    "config2": "BASELINE.json configs[2]: N=32, C=F=64, 56x56, K=3",
+    "config3": "BASELINE.json configs[3]: N=128, C=3, F=64, 224x224, K=7",
+    "config4": "BASELINE.json configs[4]: 32768x32768, K=15 (row bands + NCCL halo at N>1)",
+}
+
+
+def materialise(points, rank, world, device):
+    import torch
+
+    from gen import synth
+
+    for i, p in enumerate(points):
+        seed = synth.BASE_SEED + 1000 * rank + i
+        if p.kind == "single":
+            H, W = p.dims
+            p.x = synth.fill_torch(seed, synth.TAG_INPUT, (H, W), "img", device=device)
+            p.f = torch.from_numpy(synth.make_filter(seed, p.K, "rand")[0, 0]).to(device)
+            p.y = torch.empty((H - p.K + 1, W - p.K + 1), device=device)
+        else:
+            N, C, H, W, F = p.dims
+            p.x = synth.fill_torch(seed, synth.TAG_INPUT, (N, C, H, W), "img" if C < 8 else "sym",
+                                   device=device)
+            p.f = torch.from_numpy(synth.make_filter(seed, p.K, "he", F=F, C=C)).to(device)
+            p.y = torch.empty((N, F, H - p.K + 1, W - p.K + 1), device=device)
+
+
+# ------------------------------------------------------------------------------------------------
+# clocks (NVML, sampled in a thread during the timed region)
+# ------------------------------------------------------------------------------------------------
+class ClockSampler:
+    REASONS = {
+        "gpu_idle": 0x1, "applications_clocks_setting": 0x2, "sw_power_cap": 0x4, "hw_slowdown": 0x8,
+        "sync_boost": 0x10, "sw_thermal_slowdown": 0x20, "hw_thermal_slowdown": 0x40,
+        "hw_power_brake_slowdown": 0x80, "display_clock_setting": 0x100,
+    }
+
+    def __init__(self, index, period_s=0.01):
+        self.samples, self.reasons, self.max_mhz = [], set(), None
+        self.period = period_s
+        self._stop = threading.Event()
+        self.ok = False
+        try:
+            import pynvml
+
+            pynvml.nvmlInit()
+            self.nv = pynvml
+            self.h = pynvml.nvmlDeviceGetHandleByIndex(index)
+            self.max_mhz = pynvml.nvmlDeviceGetMaxClockInfo(self.h, pynvml.NVML_CLOCK_SM)
+            self.ok = True
+        except Exception as e:  # pragma: no cover
+            self.err = str(e)
+
+    def _run(self):
+        while not self._stop.is_set():
+            try:
+                self.samples.append(self.nv.nvmlDeviceGetClockInfo(self.h, self.nv.NVML_CLOCK_SM))
+                r = self.nv.nvmlDeviceGetCurrentClocksThrottleReasons(self.h)
+                for k, bit in self.REASONS.items():
+                    if r & bit and k != "gpu_idle":
+                        self.reasons.add(k)
+            except Exception:
+                pass
+            time.sleep(self.period)
+
+    def __enter__(self):
+        if self.ok:
+            self.t = threading.Thread(target=self._run, daemon=True)
+            self.t.start()
+        return self
+
+    def __exit__(self, *a):
+        if self.ok:
+            self._stop.set()
+            self.t.join()
+
+    def summary(self):
+        if not self.ok or not self.samples:
+            return {"sm_mhz": None, "sm_max_mhz": self.max_mhz, "reasons": [], "samples": 0}
+        return {"sm_mhz": statistics.median(self.samples), "sm_max_mhz": self.max_mhz,
+                "reasons": sorted(self.reasons), "samples": len(self.samples)}
+
+
+# ------------------------------------------------------------------------------------------------
+# GPU arm
+# ------------------------------------------------------------------------------------------------
+def run_ours(args):
+    import torch
+    import torch.distributed as dist
+
+    import paper_conf_cluster_luzw20_b200 as pkg
+    from paper_conf_cluster_luzw20_b200 import shard
+
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    if world > 1:
+        torch.cuda.set_device(local)
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    device = torch.device("cuda", local)
+    torch.cuda.set_device(device)
+    peaks = load_peaks()
+
+    points, unit = workload_points(args.workload)
+    rowband = args.workload == "config4" and world > 1
+    band = None
+    if rowband:
+        p = points[0]
+        H, W = p.dims
+        band = shard.row_band(H, W, p.K, world, rank)
+        from gen import synth
+
+        p.x = torch.empty((band.buf_rows, W), device=device)
+        p.x[:band.in_rows] = synth.fill_torch(synth.BASE_SEED, synth.TAG_INPUT, (band.in_rows, W), "img",
+                                              start=band.o0 * W, device=device)
+        p.f = torch.from_numpy(synth.make_filter(synth.BASE_SEED, p.K, "gauss")[0, 0]).to(device)
+        p.y = torch.empty((band.out_rows, W - p.K + 1), device=device)
+    else:
+        materialise(points, rank, world, device)
+    stream = torch.cuda.current_stream(device)
+    flush = torch.empty(512 * (1 << 20) // 4, dtype=torch.float32, device=device)
+
+    def run_point(p):
+        if rowband:
+            shard.rowband_conv2d_single(p.x, p.f, band, p.y)
+        elif p.kind == "single":
+            pkg.conv2d_single(p.x, p.f, out=p.y, stream=stream)
+        else:
+            pkg.conv2d_multi(p.x, p.f, out=p.y, stream=stream)
+
+    def step(evs=None):
+        for i, p in enumerate(points):
+            run_point(p)
+            if evs is not None:
+                evs[i + 1].record(stream)
+
+    for _ in range(args.warmup):
+        flush.zero_()
+        step()
+    torch.cuda.synchronize()
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+
+    n = len(points)
+    step_events = [[torch.cuda.Event(enable_timing=True) for _ in range(n + 1)] for _ in range(args.steps)]
+    with ClockSampler(local) as clk:
+        for s in range(args.steps):
+            flush.zero_()  # L2 flush, outside [ev0, evN]
+            step_events[s][0].record(stream)
+            step(step_events[s])
+        torch.cuda.synchronize()
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+
+    per_point_ms = [0.0] * n
+    total_ms = 0.0
+    for s in range(args.steps):
+        ev = step_events[s]
+        total_ms += ev[0].elapsed_time(ev[n])
+        for i in range(n):
+            per_point_ms[i] += ev[i].elapsed_time(ev[i + 1])
+    per_point_ms = [t / args.steps for t in per_point_ms]
+    if world > 1:
+        t = torch.tensor([total_ms], dtype=torch.float64, device=device)
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        total_ms = float(t.item())
+
+    units_per_step_rank = sum(p.out_px if unit == "Gpixel/s" else p.flops for p in points)
+    if rowband:
+        units_per_step = sum(p.out_px for p in points)  # the one image, split over ranks
+    else:
+        units_per_step = units_per_step_rank * world
+    value = units_per_step * args.steps / (total_ms * 1e-3) / 1e9
+
+    clocks = clk.summary()
+    sm_mhz_peak = peaks["sm_max_mhz"]
+
+    # roofline of the dominant kernel (largest share of the step)
+    dom = max(range(n), key=lambda i: per_point_ms[i])
+    dp = points[dom]
+    dkind, _ = dp.bound(peaks, sm_mhz_peak)
+    dsec = per_point_ms[dom] * 1e-3
+    if dkind == "hbm":
+        roof = {"bound": "hbm", "achieved": dp.bytes / dsec / 1e9, "peak": peaks["hbm_gbs"], "unit": "GB/s"}
+    else:
+        roof = {"bound": "alu", "achieved": dp.flops / dsec / 1e12, "peak": fp32_fma_peak_tflops(sm_mhz_peak),
+                "unit": "TFLOP/s"}
+    roof["frac"] = roof["achieved"] / roof["peak"]
+    roof["kernel"] = f"conv2d_{dp.kind} {dp.name}"
+    roof["share_of_step"] = per_point_ms[dom] / max(sum(per_point_ms), 1e-12)
+    roof["peak_source"] = (peaks["source"] if dkind == "hbm" else
+                           f"fp32 FMA: 148 SM x 128 lanes x 2 x {sm_mhz_peak:.0f} MHz (sm_max_mhz, "
+                           f"{peaks['source']})")
+    roof["traffic"] = load_traffic(dp)
+
+    sweep = []
+    for i, p in enumerate(points):
+        kind, t_roof = p.bound(peaks, sm_mhz_peak)
+        t = per_point_ms[i] * 1e-3
+        sweep.append({"point": p.name, "ms": round(per_point_ms[i], 5),
+                      ("gpx_s" if unit == "Gpixel/s" else "gflop_s"):
+                          round((p.out_px if unit == "Gpixel/s" else p.flops) / t / 1e9, 2),
+                      "bound": kind, "roofline_frac": round(t_roof / t, 4)})
+
+    line = {
+        "metric": BASELINE_METRIC,
+        "metric_detail": f"{unit} of the {args.workload} workload (whole job, all ranks)",
+        "value": round(value, 3),
+        "unit": unit,
+        "n_gpus": world,
+        "steps": args.steps,
+        "warmup": args.warmup,
+        "ms_per_step": round(total_ms / args.steps, 5),
+        "higher_is_better": True,
+        "scaling": "strong" if rowband else "weak",
+        "vs_baseline": None,
+        "dtype": "f32",
+        "data": "synthetic (seeded counter-based generator, gen/synth.py)",
+        "config": {"workload": WORKLOAD_DESC[args.workload],
+                   "l2": "512 MiB write between timed steps (outside the events) + distinct buffers per "
+                         "conv; 8192^2 inputs also exceed L2",
+                   "parallelism": ("row bands + NCCL halo" if rowband else
+                                   ("replicas (independent images per rank)" if world > 1 else "1 GPU")),
+                   "filter": "rand (2u-1)/K", "input": "img u in [0,1)"},
+        "roofline": roof,
+        "gpu_launches": n * args.steps * (2 if rowband and band is not None and not band.is_last else 1),
+        "clocks": clocks,
+        "sweep": sweep,
+    }
+
+    # end to end through the public API with host buffers (pinned), copies inside the timed region
+    if rank == 0 and not rowband and not args.no_e2e:
+        line["e2e"] = run_e2e(points, unit, args, device)
+
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+        line["cpu_baseline"] = cpu_baseline(args.workload, budget_s=args.cpu_budget)
+
+    if world > 1:
+        dist.barrier()
+        dist.destroy_process_group()
+    if rank == 0:
+        print(json.dumps(line), flush=True)
+
+
+def run_e2e(points, unit, args, device):
+    """Same metric through the user-facing host-buffer call: per conv, pinned host -> HBM copy of the
+    input and filter, the kernel, HBM -> pinned host copy of the output; all inside the events."""
+    import torch
+
+    import paper_conf_cluster_luzw20_b200 as pkg
+
+    stream = torch.cuda.current_stream(device)
+    hx = [p.x.cpu().pin_memory() for p in points]
+    hf = [p.f.cpu().pin_memory() for p in points]
+    hy = [torch.empty(tuple(p.y.shape), dtype=torch.float32, pin_memory=True) for p in points]
+    steps = max(1, min(args.steps, args.e2e_steps))
+
+    def one():
+        for i, p in enumerate(points):
+            fn = pkg.conv2d_single_host if p.kind == "single" else pkg.conv2d_multi_host
+            fn(hx[i], hf[i], device=device, stream=stream, out_host=hy[i])
+
+    one()
+    torch.cuda.synchronize()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    e0.record(stream)
+    for _ in range(steps):
+        one()
+    e1.record(stream)
+    torch.cuda.synchronize()
+    ms = e0.elapsed_time(e1)
+    units = sum(p.out_px if unit == "Gpixel/s" else p.flops for p in points) * steps
+    h2d = sum(p.in_bytes() + p.filt_bytes() for p in points)
+    d2h = sum(4 * p.y.numel() for p in points)
+    return {"value": round(units / (ms * 1e-3) / 1e9, 3), "unit": unit, "h2d_bytes_per_step": h2d,
+            "d2h_bytes_per_step": d2h, "steps": steps, "ms_per_step": round(ms / steps, 3)}
+
+
+def load_traffic(p):
+    """dram bytes (read + write) per launch of this kernel config from the committed ncu capture."""
+    path = os.path.join(ROOT, "profiles", "ncu_traffic.json")
+    try:
+        with open(path) as fh:
+            d = json.load(fh)
+        return d.get(f"conv2d_{p.kind} {p.name}")
+    except Exception:
+        return None
+
+
+# ------------------------------------------------------------------------------------------------
+# CPU oracle legs (cpu_baseline and --impl reference) -- the only bench code touching oracle/
+# ------------------------------------------------------------------------------------------------
+def _oracle_sample(points, frac):
+    """Run the oracle on the first ceil(frac * rows) output rows (single) / images (multi) of every
+    point; inputs for just those rows are generated on the host. Returns (units, seconds)."""
+    import numpy as np
+
+    import oracle
+    from gen import synth
+
+    units = 0.0
+    secs = 0.0
+    for i, p in enumerate(points):
+        seed = synth.BASE_SEED + i
+        if p.kind == "single":
+            H, W = p.dims
+            Ho = H - p.K + 1
+            rows = max(1, math.ceil(frac * Ho))
+            x = synth.fill_np(seed, synth.TAG_INPUT, (rows + p.K - 1, W), "img")
+            f = synth.make_filter(seed, p.K, "rand")[0, 0]
+            t0 = time.perf_counter()
+            oracle.conv2d_single(x, f, want_bound=False)
+            secs += time.perf_counter() - t0
+            units += rows * (W - p.K + 1)
+        else:
+            N, C, H, W, F = p.dims
+            imgs = max(1, math.ceil(frac * N))
+            x = synth.fill_np(seed, synth.TAG_INPUT, (imgs, C, H, W), "img" if C < 8 else "sym")
+            w = synth.make_filter(seed, p.K, "he", F=F, C=C)
+            t0 = time.perf_counter()
+            oracle.conv2d_multi(x, w, want_bound=False)
+            secs += time.perf_counter() - t0
+            units += 2.0 * imgs * F * (H - p.K + 1) * (W - p.K + 1) * C * p.K * p.K
+    return units, secs
+
+
+def _set_omp():
+    os.environ.setdefault("OMP_NUM_THREADS", str(len(os.sched_getaffinity(0))))
+
+
+def _calibrate(points, budget_s):
+    """Pick the sample fraction so the oracle sample takes about budget_s seconds (capped at 1)."""
+    total_rows = sum((p.dims[0] - p.K + 1) if p.kind == "single" else p.dims[0] for p in points)
+    frac = min(1.0, 2.0 * len(points) / total_rows)  # a couple of rows per point
+    u, s = _oracle_sample(points, frac)
+    while s < 0.5 and frac < 1.0:
+        frac = min(1.0, frac * 4)
+        u, s = _oracle_sample(points, frac)
+    return min(1.0, frac * budget_s / max(s, 1e-6)), u, s
+
+
+def cpu_baseline(workload, budget_s=10.0):
+    _set_omp()
+    import oracle
+
+    points, unit = workload_points(workload)
+    frac, _, _ = _calibrate(points, budget_s)
+    u, s = _oracle_sample(points, frac)
+    what = "output rows" if points[0].kind == "single" else "images"
+    return {"value": round(u / s / 1e9, 6), "unit": unit, "cores": oracle.num_threads(), "kind": "oracle",
+            "sample": f"first {frac * 100:.3g}% of the {what} of every point of the {workload} workload "
+                      f"({s:.1f} s of oracle time; double accumulation, OpenMP over output rows)",
+            "seconds": round(s, 2)}
+
+
+def run_reference(args):
+    rank = int(os.environ.get("RANK", "0"))
+    if rank != 0:
+        return  # under torchrun only rank 0 runs the CPU reference
+    _set_omp()
+    import oracle
+
+    points, unit = workload_points(args.workload)
+    budget = max(0.5, args.ref_budget / max(1, args.steps + args.warmup))
+    frac, _, _ = _calibrate(points, budget)
+    for _ in range(args.warmup):
+        _oracle_sample(points, frac)
+    tot_u = tot_s = 0.0
+    for _ in range(args.steps):
+        u, s = _oracle_sample(points, frac)
+        tot_u += u
+        tot_s += s
+    value = tot_u / tot_s / 1e9
+    what = "output rows" if points[0].kind == "single" else "images"
+    sample = (f"each step: first {frac * 100:.3g}% of the {what} of every point of the {args.workload} "
+              f"workload (bounded sample; the full step would take ~{tot_s / args.steps / frac:.0f} s)")
+    print(json.dumps({
+        "impl": "reference",
+        "metric": BASELINE_METRIC,
+        "metric_detail": f"{unit} of the {args.workload} workload, CPU oracle",
+        "value": round(value, 6), "unit": unit, "n_gpus": int(os.environ.get("WORLD_SIZE", "1")),
+        "steps": args.steps, "warmup": args.warmup, "ms_per_step": round(tot_s / args.steps * 1e3, 3),
+        "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f64",
+        "data": "synthetic (seeded counter-based generator, gen/synth.py)",
+        "config": {"workload": WORKLOAD_DESC[args.workload], "sample_fraction": frac},
+        "cpu_baseline": {"value": round(value, 6), "unit": unit, "cores": oracle.num_threads(),
+                         "kind": "oracle", "sample": sample},
+        "e2e": {"value": round(value, 6), "unit": unit, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+        "gpu_launches": 0,
+    }), flush=True)
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=20)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
+    ap.add_argument("--workload", default="sweep", choices=sorted(WORKLOAD_DESC))
+    ap.add_argument("--e2e-steps", type=int, default=2)
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--cpu-budget", type=float, default=10.0)
+    ap.add_argument("--ref-budget", type=float, default=90.0)
+    args = ap.parse_args()
+    if args.warmup < 3 and args.impl == "ours":
+        args.warmup = 3  # contract: W >= 3
+    if args.impl == "reference":
+        run_reference(args)
+    else:
+        run_ours(args)
+
+
+if __name__ == "__main__":
+    main()

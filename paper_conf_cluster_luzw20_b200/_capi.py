@@ -87,3 +87,19 @@ def conv2d_multi_ex(in_ptr, N, C, H, W, filt_ptr, F, K, out_ptr, stream=0, band_
 
 def conv2d_version() -> int:
     return load().conv2d_version()
+
+
+def debug_set_variant(v: int) -> int:
+    """Tuning hook (not in include/conv2d.h): force a single-channel kernel variant; 0 = default."""
+    L = load()
+    L.c2d_debug_set_variant.argtypes = [ctypes.c_int]
+    L.c2d_debug_set_variant.restype = ctypes.c_int
+    return L.c2d_debug_set_variant(int(v))
+
+
+def debug_set_min_band(v: int) -> int:
+    """Tuning hook (not in include/conv2d.h): minimum band height of the automatic band choice."""
+    L = load()
+    L.c2d_debug_set_min_band.argtypes = [ctypes.c_int]
+    L.c2d_debug_set_min_band.restype = ctypes.c_int
+    return L.c2d_debug_set_min_band(int(v))

@@ -48,11 +48,11 @@ int ceil_div(long long a, long long b) { return static_cast<int>((a + b - 1) / b
 // Occupancy (CTAs per SM) of a kernel instantiation, cached per instantiation (devices of one box
 // are identical B200s).
 template <typename KernelT>
-int cta_occupancy(KernelT kernel, size_t dyn_smem, std::atomic<int> &cache) {
+int cta_occupancy(KernelT kernel, size_t dyn_smem, std::atomic<int> &cache, int cta_warps = kCtaWarps) {
   int v = cache.load(std::memory_order_relaxed);
   if (v > 0) return v;
   int blocks = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, kernel, kCtaWarps * kWarp, dyn_smem) != cudaSuccess ||
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, kernel, cta_warps * kWarp, dyn_smem) != cudaSuccess ||
       blocks < 1)
     blocks = 1;
   cache.store(blocks, std::memory_order_relaxed);
@@ -62,18 +62,60 @@ int cta_occupancy(KernelT kernel, size_t dyn_smem, std::atomic<int> &cache) {
 // ------------------------------------------------------------------------------------------------
 // single channel
 // ------------------------------------------------------------------------------------------------
-template <int K>
-struct SingleCfg {
-  static constexpr int U = 1;
-  static constexpr int PF = (K <= 5) ? 4 : (K <= 9 ? 2 : 1);
-};
+// Variant override for tuning tools (c2d_debug_set_variant; 0 = the tuned default):
+//   1: filter in shared memory, U=1 (4 warps/CTA)     2: shared memory, U=2
+//   3: filter in a __constant__ slot, U=1 (1 warp/CTA) 4: __constant__ slot, U=2
+std::atomic<int> g_variant{0};
+std::atomic<int> g_min_band{0};  // tuning override of the minimum band height (0 = per-K default)
 
-template <int K>
-int launch_single(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                  const DevInfo &dev) {
-  constexpr int U = SingleCfg<K>::U;
-  constexpr int PF = SingleCfg<K>::PF;
-  auto kernel = k_conv2d_single<K, U, PF>;
+// Constant-bank filter slots, per device: slot K holds the filter of the last call with this K. A
+// call waits (stream-ordered) for the event recorded behind the previous kernel that read the slot
+// before overwriting it, so calls on different streams never see each other's filter; calls with
+// the same K on different streams are serialised by that wait, calls on one stream cost nothing.
+struct ConstRing {
+  std::mutex mu;
+  bool init = false;
+  float *base = nullptr;  // device address of c_filt
+  cudaEvent_t ev[kConstSlots];
+};
+ConstRing g_cring[kMaxDevices];
+
+template <typename LaunchFn>
+int with_const_filter(const float *filt, int K, int KP, cudaStream_t stream, LaunchFn launch) {
+  int dev = 0;
+  if (cudaGetDevice(&dev) != cudaSuccess || dev < 0 || dev >= kMaxDevices) return CONV2D_ECUDA;
+  ConstRing &ring = g_cring[dev];
+  std::lock_guard<std::mutex> lk(ring.mu);
+  if (!ring.init) {
+    void *p = nullptr;
+    if (cudaGetSymbolAddress(&p, c_filt) != cudaSuccess) return CONV2D_ECUDA;
+    ring.base = static_cast<float *>(p);
+    for (int i = 0; i < kConstSlots; ++i)
+      if (cudaEventCreateWithFlags(&ring.ev[i], cudaEventDisableTiming) != cudaSuccess) return CONV2D_ECUDA;
+    ring.init = true;
+  }
+  const int slot = K;
+  if (cudaStreamWaitEvent(stream, ring.ev[slot], 0) != cudaSuccess) return CONV2D_ECUDA;
+  // K rows of K floats -> K rows of KP floats (16-byte aligned rows for LDCU.128)
+  if (cudaMemcpy2DAsync(ring.base + static_cast<size_t>(slot) * kConstSlotFloats, KP * sizeof(float), filt,
+                        K * sizeof(float), K * sizeof(float), K, cudaMemcpyDeviceToDevice, stream) != cudaSuccess)
+    return CONV2D_ECUDA;
+  const int rc = launch();
+  if (rc != CONV2D_OK) return rc;
+  if (cudaEventRecord(ring.ev[slot], stream) != cudaSuccess) return CONV2D_ECUDA;
+  return CONV2D_OK;
+}
+
+bool stream_capturing(cudaStream_t s) {
+  cudaStreamCaptureStatus st = cudaStreamCaptureStatusNone;
+  return cudaStreamIsCapturing(s, &st) == cudaSuccess && st != cudaStreamCaptureStatusNone;
+}
+
+template <int K, int U, int FSRC, int PF = 1, int GUARDS = 0>
+int launch_single_v(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
+                    const DevInfo &dev, int min_band) {
+  constexpr int CTAW = (FSRC == FSRC_CONST) ? 1 : kCtaWarps;
+  auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS>;
   static std::atomic<int> occ_cache{0};
   SingleArgs a;
   a.in = in;
@@ -86,20 +128,54 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
   a.n_cb = ceil_div(a.Wo, 128 * U);
   a.aligned = (aligned16(in) && (W % 4 == 0)) ? 1 : 0;
   if (band_h <= 0) {
-    const long long resident_warps = static_cast<long long>(cta_occupancy(kernel, 0, occ_cache)) * kCtaWarps *
-                                     dev.num_sms;
+    // one full wave of warp tiles: bands = resident warps / column blocks
+    const long long resident_warps =
+        static_cast<long long>(cta_occupancy(kernel, 0, occ_cache, CTAW)) * CTAW * dev.num_sms;
     const long long bands = resident_warps / a.n_cb > 0 ? resident_warps / a.n_cb : 1;
     band_h = ceil_div(a.Ho, bands);
-    const int min_band = 8;
     if (band_h < min_band) band_h = min_band;
   }
   if (band_h > a.Ho) band_h = a.Ho;
   a.band_h = band_h;
   const int n_bands = ceil_div(a.Ho, band_h);
   a.n_tiles = a.n_cb * n_bands;
-  const int blocks = ceil_div(a.n_tiles, kCtaWarps);
-  kernel<<<blocks, kCtaWarps * kWarp, 0, stream>>>(a);
-  return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
+  const int blocks = ceil_div(a.n_tiles, CTAW);
+  auto go = [&]() {
+    kernel<<<blocks, CTAW * kWarp, 0, stream>>>(a);
+    return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
+  };
+  if constexpr (FSRC == FSRC_CONST) return with_const_filter(filt, K, KCfg<K>::KP, stream, go);
+  return go();
+}
+
+template <int K>
+int launch_single(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
+                  const DevInfo &dev) {
+  const int mb = g_min_band.load(std::memory_order_relaxed);
+  const int min_band = mb > 0 ? mb : (K - 1 > 4 ? K - 1 : 4);
+  const int v = g_variant.load(std::memory_order_relaxed);
+  // CUDA-graph capture cannot use the event-guarded constant slots: shared-memory filter there
+  const bool constant_ok = !stream_capturing(stream);
+#define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G>(in, H, W, filt, out, stream, band_h, dev, min_band)
+  switch (v) {
+    case 1: return C2D_LS(1, FSRC_SMEM, 1, 0);
+    case 2: return C2D_LS(2, FSRC_SMEM, 1, 0);
+    case 3: if (constant_ok) return C2D_LS(1, FSRC_CONST, 1, 0); break;
+    case 4: if (constant_ok) return C2D_LS(2, FSRC_CONST, 1, 0); break;
+    case 5: if (constant_ok) return C2D_LS(1, FSRC_CONST, 1, 1); break;
+    case 6: if (constant_ok) return C2D_LS(1, FSRC_CONST, 1, 2); break;
+    default: break;
+  }
+  // Tuned on B200 (tools/variants.py, profiles/): two 128-column
+  // chunks per warp while K <= 7 (K = 9 on wide images); above, one chunk with a guarded prologue on
+  // wide images (tall bands) and guarded prologue + epilogue on narrow ones (short bands, where the
+  // wasted FMAs of an unguarded epilogue would be a large fraction).
+  const bool u2 = (K <= 7) || (K <= 9 && W > 3000);
+  if (!constant_ok) return u2 ? C2D_LS(2, FSRC_SMEM, 1, 0) : C2D_LS(1, FSRC_SMEM, 1, 0);
+  if (u2) return C2D_LS(2, FSRC_CONST, 1, 0);
+  if (W >= 4096) return C2D_LS(1, FSRC_CONST, 1, 1);
+  return C2D_LS(1, FSRC_CONST, 1, 2);
+#undef C2D_LS
 }
 
 // ------------------------------------------------------------------------------------------------
@@ -285,5 +361,17 @@ const char *conv2d_strerror(int code) {
 }
 
 int conv2d_version(void) { return 100; }
+
+// Not part of include/conv2d.h: selects a kernel variant for tuning tools (0 = default).
+int c2d_debug_set_variant(int v) {
+  const int old = g_variant.exchange(v);
+  return old;
+}
+
+// Not part of include/conv2d.h: minimum band height override for tuning tools (0 = default).
+int c2d_debug_set_min_band(int v) {
+  const int old = g_min_band.exchange(v);
+  return old;
+}
 
 }  // extern "C"

@@ -5,9 +5,9 @@
 //   * One WARP owns a tile of 128*U output columns x BH output rows ("band"). Lane l holds the
 //     outputs x0 + 128u + 4l + {0..3} of every chunk u < U (V = 4 contiguous columns per lane, so
 //     every input-row load is one coalesced LDG.128 per lane and every output store is STG.128).
-//   * a1 Input row fetch: per input row, U LDG.128 per lane plus one extra LDG.128 on the first
-//     NE = ceil((K-1)/4) lanes (the K-1 halo columns right of the warp's span). Rows are prefetched
-//     PF rows ahead in registers.
+//   * a1 Input row fetch: per input row, U LDG.128 per lane plus one extra LDG.128 for the K-1 halo
+//     columns right of the warp's span (lanes >= NE = ceil((K-1)/4) re-read a duplicate quad so the
+//     load is branch-free). The next row is in flight while the current one is computed.
 //   * a2 Column reuse (Sec. II-A, Alg. 1, Fig. 1c): the K-1 halo values
 //     a lane needs beyond its own 4 come from lanes l+1.. via __shfl_sync, never from memory. As in
 //     Alg. 1, the value a lane SUPPLIES is chosen with a static register index and a lane-dependent
@@ -22,9 +22,9 @@
 //     static (the dynamic->static index transformation of P:75-77). The first K-1 rows
 //     of a band (Alg. 2 case 1) skip the slots whose output row precedes the band; Alg. 2 case 3 is
 //     implicit (the band stops when its last output row completes).
-//   * a4 Filter supply: the CTA stages the filter into shared memory once (rows padded to KP floats)
-//     and the FMAs read it with broadcast LDS.128 (or from registers for K <= 5). Reentrant: no
-//     __constant__ state.
+//   * a4 Filter supply: a per-launch slot of the __constant__ bank read through uniform registers
+//     (LDCU.128 + FFMA with a UR operand: one fetch serves the whole warp, no per-lane traffic), or
+//     shared memory (broadcast LDS.128) when the launch is being captured into a CUDA graph.
 //   * a5 Channel reduction (multi): for each input row, all C channels stream through the same
 //     accumulators; each thread also carries FB filters, so one window feeds FB*K*K*4 FMAs.
 //   * a6 Output store: slot 0 is complete after each row -> one coalesced store per lane; rows whose
@@ -58,8 +58,8 @@ __device__ __forceinline__ void stg4(float *p, float a, float b, float c, float 
   __stcs(reinterpret_cast<float4 *>(p), make_float4(a, b, c, d));
 }
 
-// LDS.128 that the compiler may not hoist out of the row loop (keeps K*K filter values out of the
-// register file for large K).
+// LDS.128 that the compiler may not hoist out of the row loop (keeps the staged filters out of the
+// register file).
 __device__ __forceinline__ void lds4_volatile(const float *p, float &a, float &b, float &c, float &d) {
   const unsigned s = static_cast<unsigned>(__cvta_generic_to_shared(p));
   asm volatile("ld.shared.v4.f32 {%0, %1, %2, %3}, [%4];" : "=f"(a), "=f"(b), "=f"(c), "=f"(d) : "r"(s));
@@ -89,14 +89,19 @@ __device__ __forceinline__ void load_row(RowBuf<K, U> &b, const float *__restric
       for (int t = 0; t < 4; ++t) b.a[u][t] = (x + t < W) ? __ldg(rowp + x + t) : 0.f;
     }
   }
+  if constexpr (KCfg<K>::NE == 0) {
 #pragma unroll
-  for (int t = 0; t < 4; ++t) b.e[t] = 0.f;
-  if (KCfg<K>::NE > 0 && lane < KCfg<K>::NE) {
-    const int x = x0 + 128 * U + 4 * lane;
-    if (!SAFE && x + 3 < W) {
-      const float4 v = ldg4(rowp + x);
-      b.e[0] = v.x; b.e[1] = v.y; b.e[2] = v.z; b.e[3] = v.w;
-    } else {
+    for (int t = 0; t < 4; ++t) b.e[t] = 0.f;
+  } else if constexpr (!SAFE) {
+    // fast tiles guarantee x0 + 128U + 4*NE <= W: every lane loads (lanes >= NE re-read lane
+    // (l mod NE)'s quad, same sectors), no branch
+    const float4 v = ldg4(rowp + x0 + 128 * U + 4 * (lane % KCfg<K>::NE));
+    b.e[0] = v.x; b.e[1] = v.y; b.e[2] = v.z; b.e[3] = v.w;
+  } else {
+#pragma unroll
+    for (int t = 0; t < 4; ++t) b.e[t] = 0.f;
+    if (lane < KCfg<K>::NE) {
+      const int x = x0 + 128 * U + 4 * lane;
 #pragma unroll
       for (int t = 0; t < 4; ++t) b.e[t] = (x + t < W) ? __ldg(rowp + x + t) : 0.f;
     }
@@ -130,20 +135,52 @@ __device__ __forceinline__ void build_windows(const RowBuf<K, U> &b, float (&w)[
 }
 
 // ------------------------------------------------------------------------------------------------
-// a4: filter row i as K registers
+// a4: filter supply. A filter row i is fetched into K registers right before the FMAs that use it:
+//   FSRC_CONST -- the __constant__ slot of this K (slot K, rows padded to KP floats), staged by the
+//                 host with a stream-ordered 2D device-to-device copy; a call waits (stream-ordered,
+//                 on a CUDA event) for the previous kernel that read the slot, so calls on other
+//                 streams never see each other's filter. The slot address is a compile-time constant
+//                 and the control flow is warp-uniform (one warp per CTA), so the compiler reads the
+//                 filter with LDCU.128 into uniform registers and feeds FFMA's UR operand: one
+//                 16-byte fetch per warp, no per-lane return traffic through the LSU/MIO path.
+//   FSRC_SMEM  -- staged per CTA in shared memory (rows padded to KP floats), broadcast LDS.128. Each
+//                 LDS.128 still returns 512 B through the shared-memory crossbar (16 B x 32 lanes),
+//                 which caps large-K FMA throughput (profiles/); used when a launch is captured into
+//                 a CUDA graph (the constant-slot recycling needs stream-ordered events).
 // ------------------------------------------------------------------------------------------------
-template <int K, bool FREG>
-__device__ __forceinline__ void filter_row(float (&fr)[KCfg<K>::KP], const float *__restrict__ sf_row,
-                                           const float (&freg)[FREG ? K * K : 1], int i) {
-  if constexpr (FREG) {
-#pragma unroll
-    for (int j = 0; j < K; ++j) fr[j] = freg[i * K + j];
-  } else {
-#pragma unroll
-    for (int c = 0; c < KCfg<K>::KP / 4; ++c)
-      lds4_volatile(sf_row + 4 * c, fr[4 * c], fr[4 * c + 1], fr[4 * c + 2], fr[4 * c + 3]);
-  }
+constexpr int FSRC_SMEM = 0;
+constexpr int FSRC_CONST = 1;
+
+constexpr int kConstSlotFloats = 256;  // >= 15 rows x 16 (padded) floats
+constexpr int kConstSlots = 16;        // slot K for K = 1..15 (16 KiB of the 64 KiB constant bank)
+__constant__ __align__(16) float c_filt[kConstSlots * kConstSlotFloats];
+
+__device__ __forceinline__ void lds4_at(unsigned saddr, float &a, float &b, float &c, float &d) {
+  asm volatile("ld.shared.v4.f32 {%0, %1, %2, %3}, [%4];" : "=f"(a), "=f"(b), "=f"(c), "=f"(d) : "r"(saddr));
 }
+
+template <int K, int FSRC>
+struct FilterSrc {
+  unsigned sbase;      // FSRC_SMEM: shared-window address of row 0
+  const float *cbase;  // FSRC_CONST: slot K of c_filt (compile-time address, rows of KP floats)
+
+  __device__ __forceinline__ void row(float (&fr)[KCfg<K>::KP], int i) const {
+    constexpr int KP = KCfg<K>::KP;
+    if constexpr (FSRC == FSRC_CONST) {
+      const float4 *p = reinterpret_cast<const float4 *>(cbase + i * KP);
+#pragma unroll
+      for (int c = 0; c < KP / 4; ++c) {
+        const float4 v = p[c];
+        fr[4 * c] = v.x; fr[4 * c + 1] = v.y; fr[4 * c + 2] = v.z; fr[4 * c + 3] = v.w;
+      }
+    } else {
+#pragma unroll
+      for (int c = 0; c < KP / 4; ++c)
+        lds4_at(sbase + static_cast<unsigned>((i * KP + 4 * c) * 4), fr[4 * c], fr[4 * c + 1], fr[4 * c + 2],
+                fr[4 * c + 3]);
+    }
+  }
+};
 
 // ------------------------------------------------------------------------------------------------
 // a6: store 4 outputs per lane of a 128-wide output chunk starting at g (16B alignment unknown)
@@ -199,23 +236,26 @@ __device__ __forceinline__ void store_row(float *__restrict__ orow, int x0, int 
 }
 
 // ------------------------------------------------------------------------------------------------
-// a3: row reuse -- one input row into the K-slot accumulator ring (single channel)
+// a3: row reuse (single channel). acc[q] holds output row r-K+1+q after input row r.
 // ------------------------------------------------------------------------------------------------
-template <int K, int U, bool FREG>
-__device__ __forceinline__ void row_reuse_single(float (&acc)[K][U][4], const float (&w)[U][KCfg<K>::WN],
-                                                 const float *__restrict__ sf,
-                                                 const float (&freg)[FREG ? K * K : 1], int qmin) {
+// One input row (windows w) into the ring: acc[q] = acc[q+1] + w . filter[K-1-q]. The ring shift is
+// folded into the first FMA of each chain (no MOVs); per output the terms arrive in filter-row,
+// filter-column order, independent of where the band starts (band-independent bits). GUARD: only
+// slots qmin <= q < qmax -- the first K-1 rows of a band feed fewer of its outputs (Alg. 2 case 1),
+// and so do the last K-1 (case 3); the branches are warp-uniform.
+template <int K, int U, int FSRC, bool GUARD>
+__device__ __forceinline__ void row_step1(float (&acc)[K][U][4], const float (&w)[U][KCfg<K>::WN],
+                                          const FilterSrc<K, FSRC> &fs, int qmin, int qmax) {
 #pragma unroll
   for (int q = 0; q < K; ++q) {
-    if (q >= qmin) {  // warp-uniform: the first K-1 rows of a band feed fewer outputs (Alg. 2 case 1)
-      const int i = K - 1 - q;  // filter row that input row r contributes to output row r-K+1+q
+    if (!GUARD || (q >= qmin && q < qmax)) {
       float fr[KCfg<K>::KP];
-      filter_row<K, FREG>(fr, sf + i * KCfg<K>::KP, freg, i);
+      fs.row(fr, K - 1 - q);
 #pragma unroll
       for (int u = 0; u < U; ++u) {
 #pragma unroll
         for (int v = 0; v < 4; ++v) {
-          float s = (q + 1 < K) ? acc[(q + 1 < K) ? q + 1 : 0][u][v] : 0.f;  // ring shift
+          float s = (q + 1 < K) ? acc[(q + 1 < K) ? q + 1 : 0][u][v] : 0.f;
 #pragma unroll
           for (int j = 0; j < K; ++j) s = fmaf(w[u][v + j], fr[j], s);
           acc[q][u][v] = s;
@@ -239,18 +279,31 @@ struct SingleArgs {
   int aligned;    // in is 16B aligned and W % 4 == 0
 };
 
-template <int K, int U, int PF, bool SAFE>
-__device__ __forceinline__ void single_tile(const SingleArgs &a, const float *__restrict__ sf,
-                                            const float (&freg)[(K <= 5) ? K * K : 1], int x0, int ob, int oe,
-                                            int lane) {
-  constexpr bool FREG = (K <= 5);
-  const int rend = oe + K - 1;  // input rows [ob, rend)
-  const float *__restrict__ in = a.in;
-  RowBuf<K, U> buf[PF];
-#pragma unroll
-  for (int p = 0; p < PF; ++p)
-    if (ob + p < rend) load_row<K, U, SAFE>(buf[p], in + static_cast<size_t>(ob + p) * a.W, x0, a.W, lane);
+__device__ __forceinline__ const float *in_row(const SingleArgs &a, int r) {
+  return a.in + static_cast<size_t>(r) * a.W;
+}
+__device__ __forceinline__ float *out_row(const SingleArgs &a, int o) {
+  return a.out + static_cast<size_t>(o) * a.Wo;
+}
 
+// One warp tile: 128*U columns x output rows [ob, oe). Input rows [ob, oe+K-1) stream through once,
+// following Algorithm 2's three cases: the first K-1 rows feed only the slots of outputs
+// >= ob (case 1, no stores), the steady state feeds all K slots and completes one output row per
+// input row (case 2), the last K-1 rows feed only outputs < oe (case 3, fixed per DESIGN.md R8).
+// GUARDS selects how cases 1 and 3 are run:
+//   0 -- one loop, every row runs the full K-slot body (the extra FMAs of cases 1/3 land in slots that
+//        are never stored): a single hot loop, no per-slot branches (best I-cache / scheduling);
+//   1 -- case 1 in its own loop with per-slot warp-uniform branches, cases 2+3 unguarded;
+//   2 -- cases 1 and 3 both guarded (no wasted FMA, but the per-slot branches split the FMA stream
+//        into basic blocks the scheduler cannot overlap).
+// Row r+1 (r+2 when PF == 2) is in flight from memory while row r is computed; the next-row index
+// is clamped, so the loop body has no branch besides the store.
+template <int K, int U, int FSRC, int PF, int GUARDS, bool SAFE>
+__device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc<K, FSRC> &fs, int x0, int ob,
+                                            int oe, int lane) {
+  static_assert(PF == 1 || PF == 2, "prefetch depth 1 or 2 rows");
+  const int rend = oe + K - 1;  // input rows [ob, rend)
+  const int rlast = rend - 1;
   float acc[K][U][4];
 #pragma unroll
   for (int q = 0; q < K; ++q)
@@ -258,62 +311,87 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const float *__
     for (int u = 0; u < U; ++u)
 #pragma unroll
       for (int v = 0; v < 4; ++v) acc[q][u][v] = 0.f;
-
-  for (int r0 = ob; r0 < rend; r0 += PF) {
-#pragma unroll
-    for (int p = 0; p < PF; ++p) {
-      const int r = r0 + p;
-      if (r < rend) {
-        RowBuf<K, U> cur = buf[p];
-        if (r + PF < rend)
-          load_row<K, U, SAFE>(buf[p], in + static_cast<size_t>(r + PF) * a.W, x0, a.W, lane);
-        float w[U][KCfg<K>::WN];
-        build_windows<K, U>(cur, w, lane);
-        const int done = r - ob;  // rows of this band already streamed
-        const int qmin = (done < K - 1) ? (K - 1 - done) : 0;
-        row_reuse_single<K, U, FREG>(acc, w, sf, freg, qmin);
-        if (done >= K - 1) {  // slot 0 now holds the complete output row r-K+1
-          const float(&o)[U][4] = acc[0];
-          store_row<U, SAFE>(a.out + static_cast<size_t>(r - K + 1) * a.Wo, x0, a.Wo, o, lane);
-        }
-      }
+  RowBuf<K, U> n1, n2;  // rows r+1 (and r+2 when PF == 2) in flight
+  load_row<K, U, SAFE>(n1, in_row(a, ob), x0, a.W, lane);
+  if (PF == 2) load_row<K, U, SAFE>(n2, in_row(a, min(ob + 1, rlast)), x0, a.W, lane);
+  // advance the in-flight rows: returns row r, issues the load of row r+PF (index clamped)
+  auto next_row = [&](int r) {
+    const RowBuf<K, U> cur = n1;
+    if constexpr (PF == 2) {
+      n1 = n2;
+      load_row<K, U, SAFE>(n2, in_row(a, min(r + 2, rlast)), x0, a.W, lane);
+    } else {
+      load_row<K, U, SAFE>(n1, in_row(a, min(r + 1, rlast)), x0, a.W, lane);
     }
+    return cur;
+  };
+  int r = ob;
+  if constexpr (GUARDS == 0) {
+    for (; r < rend; ++r) {
+      const RowBuf<K, U> cur = next_row(r);
+      float w[U][KCfg<K>::WN];
+      build_windows<K, U>(cur, w, lane);
+      row_step1<K, U, FSRC, false>(acc, w, fs, 0, K);
+      if (r >= ob + K - 1) store_row<U, SAFE>(out_row(a, r - K + 1), x0, a.Wo, acc[0], lane);
+    }
+    return;
+  }
+  for (; r < min(ob + K - 1, oe); ++r) {  // case 1: slots of outputs >= ob only
+    const RowBuf<K, U> cur = next_row(r);
+    float w[U][KCfg<K>::WN];
+    build_windows<K, U>(cur, w, lane);
+    row_step1<K, U, FSRC, true>(acc, w, fs, K - 1 - (r - ob), K);
+  }
+  const int steady_end = (GUARDS == 2) ? oe : rend;
+  for (; r < steady_end; ++r) {  // case 2 (+3 when GUARDS == 1): all K slots
+    const RowBuf<K, U> cur = next_row(r);
+    float w[U][KCfg<K>::WN];
+    build_windows<K, U>(cur, w, lane);
+    row_step1<K, U, FSRC, false>(acc, w, fs, 0, K);
+    if (GUARDS == 2 || r >= ob + K - 1) store_row<U, SAFE>(out_row(a, r - K + 1), x0, a.Wo, acc[0], lane);
+  }
+  for (; r < rend; ++r) {  // case 3 (GUARDS == 2): slots of outputs < oe only (>= ob for short bands)
+    const RowBuf<K, U> cur = next_row(r);
+    float w[U][KCfg<K>::WN];
+    build_windows<K, U>(cur, w, lane);
+    row_step1<K, U, FSRC, true>(acc, w, fs, max(0, K - 1 - (r - ob)), oe + K - 1 - r);
+    if (r >= ob + K - 1) store_row<U, SAFE>(out_row(a, r - K + 1), x0, a.Wo, acc[0], lane);
   }
 }
 
-template <int K, int U, int PF>
-__global__ void __launch_bounds__(kCtaWarps *kWarp) k_conv2d_single(const SingleArgs a) {
+// CTAW: warps per CTA. With CTAW == 1 every branch depends only on blockIdx and kernel parameters,
+// so the compiler can prove warp-uniform control flow and keep the constant-bank filter in uniform
+// registers (LDCU + FFMA with UR operands) instead of per-lane loads.
+template <int K, int U, int FSRC, int CTAW, int PF = 1, int GUARDS = 0>
+__global__ void __launch_bounds__(CTAW *kWarp) k_conv2d_single(const SingleArgs a) {
   constexpr int KP = KCfg<K>::KP;
-  constexpr bool FREG = (K <= 5);
-  __shared__ __align__(16) float sf[K * KP];
-  for (int t = threadIdx.x; t < K * KP; t += blockDim.x) {
-    const int i = t / KP, j = t % KP;
-    sf[t] = (j < K) ? a.filt[i * K + j] : 0.f;
-  }
-  __syncthreads();
-  float freg[FREG ? K * K : 1];
-  if constexpr (FREG) {
-#pragma unroll
-    for (int i = 0; i < K; ++i)
-#pragma unroll
-      for (int j = 0; j < K; ++j) freg[i * K + j] = sf[i * KP + j];
+  __shared__ __align__(16) float sf[(FSRC == FSRC_SMEM) ? K * KP : 4];
+  FilterSrc<K, FSRC> fs;
+  if constexpr (FSRC == FSRC_CONST) {
+    fs.cbase = c_filt + K * kConstSlotFloats;
   } else {
-    freg[0] = 0.f;
+    for (int t = threadIdx.x; t < K * KP; t += blockDim.x) {
+      const int i = t / KP, j = t % KP;
+      sf[t] = (j < K) ? a.filt[i * K + j] : 0.f;
+    }
+    __syncthreads();
+    fs.sbase = static_cast<unsigned>(__cvta_generic_to_shared(sf));
   }
-
   const int lane = threadIdx.x & (kWarp - 1);
-  const int tile = blockIdx.x * kCtaWarps + (threadIdx.x >> 5);
+  const int tile = (CTAW == 1) ? static_cast<int>(blockIdx.x)
+                               : static_cast<int>(blockIdx.x) * CTAW + static_cast<int>(threadIdx.x >> 5);
   if (tile >= a.n_tiles) return;
   const int cb = tile % a.n_cb;
   const int band = tile / a.n_cb;
   const int x0 = cb * 128 * U;
   const int ob = band * a.band_h;
   const int oe = min(ob + a.band_h, a.Ho);
-  const bool fast = a.aligned && (x0 + 128 * U <= a.Wo);  // warp-uniform
+  // fast tiles: 16B-aligned rows, every column of the tile and its extra halo quad in range
+  const bool fast = a.aligned && (x0 + 128 * U + 4 * KCfg<K>::NE <= a.W);  // warp-uniform
   if (fast)
-    single_tile<K, U, PF, false>(a, sf, freg, x0, ob, oe, lane);
+    single_tile<K, U, FSRC, PF, GUARDS, false>(a, fs, x0, ob, oe, lane);
   else
-    single_tile<K, U, PF, true>(a, sf, freg, x0, ob, oe, lane);
+    single_tile<K, U, FSRC, PF, GUARDS, true>(a, fs, x0, ob, oe, lane);
 }
 
 // ------------------------------------------------------------------------------------------------
@@ -446,7 +524,7 @@ __global__ void __launch_bounds__(kCtaWarps *kWarp) k_conv2d_multi(const MultiAr
   const int ob = band * a.band_h;
   const int oe = min(ob + a.band_h, a.Ho);
   if (ob >= a.Ho) return;
-  const bool fast = a.aligned && (x0 + 128 <= a.Wo);
+  const bool fast = a.aligned && (x0 + 128 + 4 * KCfg<K>::NE <= a.W);
   if (fast)
     multi_tile<K, FB, false>(a, smem, n, f0, x0, ob, oe, lane);
   else

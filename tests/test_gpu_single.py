@@ -166,3 +166,69 @@ def test_config4_32768_k15_sampled(cuda_device):
         lo, hi = max(o0, o1 - 3), o1
         part = pkg.conv2d_single(x[lo:hi + K - 1], f)
         assert torch.equal(part, y[lo:hi])
+
+
+@pytest.mark.parametrize("variant", [1, 2, 3, 4, 5, 6])
+def test_every_kernel_variant_bitwise_equal(cuda_device, variant):
+    """Every instantiation (filter in shared / constant memory, 1 or 2 column chunks, guarded or
+    unguarded band prologue/epilogue) gives the same bits as the default, and passes the oracle."""
+    shapes = [(40, 300), (77, 1030), (300, 517)]
+    try:
+        for K in (1, 2, 3, 5, 8, 9, 12, 15):
+            f = _filt(K, "rand", seed=K)
+            for (dh, W) in shapes:
+                x = dev_image((K + dh, W), "img", seed=K * 7 + W)
+                _capi.debug_set_variant(0)
+                ref = pkg.conv2d_single(x, f)
+                _capi.debug_set_variant(variant)
+                got = pkg.conv2d_single(x, f)
+                torch.cuda.synchronize()
+                assert torch.equal(got, ref), (variant, K, dh, W)
+                if W == 300:
+                    check_full_single(x, f, got)
+                for bh in (1, 3, K + 1):
+                    assert torch.equal(pkg.conv2d_single(x, f, band_h=bh), ref), (variant, K, bh)
+    finally:
+        _capi.debug_set_variant(0)
+
+
+def test_cuda_graph_capture_and_replay(cuda_device):
+    """Calls captured into a CUDA graph (shared-memory filter path) replay correctly, and filters
+    updated between replays are picked up (the graph reads the filter tensor at replay time)."""
+    x = dev_image((300, 700), "img")
+    f = _filt(7)
+    y = torch.empty((294, 694), device=DEV)
+    s = torch.cuda.Stream()
+    s.wait_stream(torch.cuda.current_stream())
+    with torch.cuda.stream(s):
+        pkg.conv2d_single(x, f, out=y)  # warm-up outside capture
+    torch.cuda.current_stream().wait_stream(s)
+    g = torch.cuda.CUDAGraph()
+    with torch.cuda.graph(g):
+        pkg.conv2d_single(x, f, out=y)
+    g.replay()
+    torch.cuda.synchronize()
+    check_full_single(x, f, y)
+    f.copy_(_filt(7, "gauss"))
+    x.copy_(dev_image((300, 700), "sym", seed=9))
+    g.replay()
+    torch.cuda.synchronize()
+    check_full_single(x, f, y)
+
+
+def test_concurrent_streams_different_filters(cuda_device):
+    """Calls with the same K on two streams with different filters never see each other's filter
+    (constant-slot reuse is ordered by events)."""
+    x = dev_image((2000, 2048), "img")
+    fs = [_filt(15, "rand", seed=s) for s in range(6)]
+    outs = [torch.empty((1986, 2034), device=DEV) for _ in fs]
+    streams = [torch.cuda.Stream() for _ in range(3)]
+    for s in streams:
+        s.wait_stream(torch.cuda.current_stream())
+    for i, f in enumerate(fs):
+        st = streams[i % 3]
+        with torch.cuda.stream(st):
+            pkg.conv2d_single(x, f, out=outs[i], stream=st)
+    torch.cuda.synchronize()
+    for f, y in zip(fs, outs):
+        assert torch.equal(y, pkg.conv2d_single(x, f))
