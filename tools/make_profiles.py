@@ -1,0 +1,92 @@
+#!/usr/bin/env python
+"""Turn one measurement batch (tools/gpu_round.sh output in gpurun_out/) into the committed evidence
+under profiles/:
+
+    profiles/<tag>_bench.json             the bench.py JSON line
+    profiles/<tag>_launches.csv           ncu launch list of `bench.py --steps 2 --warmup 3` (our kernels)
+    profiles/<tag>_launch_shares.txt      per-kernel share of the timed steps (cold-cache, serialised)
+    profiles/<tag>_ncu_<name>.txt         ncu --set full summaries (key metrics + stall breakdown)
+    profiles/ncu_traffic.json             dram bytes (read + write) per launch, by bench point name
+
+    python tools/make_profiles.py <tag> [gpurun_out]
+"""
+import csv
+import io
+import json
+import os
+import re
+import sys
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, os.path.join(ROOT, "tools"))
+import ncu_raw_summary  # noqa: E402
+
+# ncu capture name -> bench point name (tools/gpu_round.sh profiles these configurations)
+CAPTURES = {
+    "prof_k15_v0_s8192": "conv2d_single 8192^2 K=15",
+    "prof_k3_v0_s8192": "conv2d_single 8192^2 K=3",
+    "prof_direct_k3_s8192": "conv2d_single_direct 8192^2 K=3 (Fig. 1a baseline)",
+}
+
+
+def launches(path, out_csv, out_txt):
+    text = open(path).read()
+    lines = [ln for ln in text.splitlines() if ln.startswith('"')]
+    rows = list(csv.reader(io.StringIO("\n".join(lines))))
+    hdr = rows[0]
+    ik, iv, ig = hdr.index("Kernel Name"), hdr.index("Metric Value"), hdr.index("Grid Size")
+    ours = [(r[ik], r[ig], float(r[iv].replace(",", ""))) for r in rows[1:] if "conv2d" in r[ik]]
+    with open(out_csv, "w") as fh:
+        w = csv.writer(fh)
+        w.writerow(["kernel", "grid", "gpu__time_duration.sum (ns)"])
+        for k, g, t in ours:
+            w.writerow([k, g, t])
+    # the last 2 steps of 28 launches are the timed ones
+    timed = ours[-56:] if len(ours) >= 56 else ours
+    tot = sum(t for _, _, t in timed)
+    by = {}
+    for k, g, t in timed:
+        key = re.sub(r"\s+", " ", k)
+        by.setdefault((key, g), []).append(t)
+    with open(out_txt, "w") as fh:
+        fh.write(f"ncu launch list (cold-cache, serialised): {len(timed)} launches of 2 timed steps, "
+                 f"total {tot / 1e3:.1f} us\n")
+        for (k, g), ts in sorted(by.items(), key=lambda kv: -sum(kv[1])):
+            fh.write(f"{100 * sum(ts) / tot:6.2f}%  {sum(ts) / len(ts) / 1e3:9.2f} us/launch  x{len(ts)}  grid {g}  {k}\n")
+
+
+def main():
+    tag = sys.argv[1]
+    src = sys.argv[2] if len(sys.argv) > 2 else os.path.join(ROOT, "gpurun_out")
+    dst = os.path.join(ROOT, "profiles")
+    os.makedirs(dst, exist_ok=True)
+    b = os.path.join(src, f"bench_{tag}.json")
+    if os.path.exists(b):
+        line = open(b).read().strip().splitlines()[-1]
+        json.loads(line)
+        open(os.path.join(dst, f"{tag}_bench.json"), "w").write(line + "\n")
+    lfile = os.path.join(src, f"launches_{tag}.csv")
+    if os.path.exists(lfile):
+        launches(lfile, os.path.join(dst, f"{tag}_launches.csv"), os.path.join(dst, f"{tag}_launch_shares.txt"))
+    traffic_path = os.path.join(dst, "ncu_traffic.json")
+    traffic = json.load(open(traffic_path)) if os.path.exists(traffic_path) else {}
+    for cap, point in CAPTURES.items():
+        raw = os.path.join(src, f"{cap}.raw.csv")
+        if not os.path.exists(raw):
+            continue
+        s = ncu_raw_summary.summary(raw)[0]
+        with open(os.path.join(dst, f"{tag}_ncu_{cap}.txt"), "w") as fh:
+            fh.write(f"# ncu --set full --clock-control none, {point}\n")
+            for k, v in s.items():
+                fh.write(f"{k}: {v}\n")
+        rd = float(s["dram__bytes_read.sum"].split()[0].replace(",", ""))
+        wr = float(s["dram__bytes_write.sum"].split()[0].replace(",", ""))
+        unit = s["dram__bytes_read.sum"].split()[1]
+        scale = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9}[unit]
+        traffic[point] = round((rd + wr) * scale)
+    json.dump(traffic, open(traffic_path, "w"), indent=1)
+    print("profiles written:", sorted(os.listdir(dst)))
+
+
+if __name__ == "__main__":
+    main()
