@@ -103,3 +103,11 @@ def debug_set_min_band(v: int) -> int:
     L.c2d_debug_set_min_band.argtypes = [ctypes.c_int]
     L.c2d_debug_set_min_band.restype = ctypes.c_int
     return L.c2d_debug_set_min_band(int(v))
+
+
+def debug_set_multi_variant(v: int) -> int:
+    """Tuning hook (not in include/conv2d.h): force a multi-channel kernel variant; 0 = default."""
+    L = load()
+    L.c2d_debug_set_multi_variant.argtypes = [ctypes.c_int]
+    L.c2d_debug_set_multi_variant.restype = ctypes.c_int
+    return L.c2d_debug_set_multi_variant(int(v))

@@ -1,0 +1,31 @@
+// common.h -- declarations shared by the C-ABI unit (conv2d_capi.cu) and the per-K launch units
+// (inst_kNN.cu): device info, tuning overrides, and the per-K launch entry points.
+#pragma once
+
+#include <atomic>
+
+#include <cuda_runtime.h>
+
+#include "../../include/conv2d.h"
+
+namespace c2d {
+
+struct DevInfo {
+  int num_sms = 0;
+  int smem_optin = 0;
+};
+
+// tuning overrides (tools/, tests): 0 = tuned default
+extern std::atomic<int> g_variant;    // single-channel kernel variant
+extern std::atomic<int> g_min_band;   // minimum band height of the automatic band choice
+extern std::atomic<int> g_mvariant;   // multi-channel kernel variant
+
+// per-K entry points, explicitly instantiated one K per translation unit (csrc/inst_kNN.cu)
+template <int K>
+int single_entry(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
+                 const DevInfo &dev);
+template <int K>
+int multi_entry(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
+                cudaStream_t stream, int band_h, const DevInfo &dev);
+
+}  // namespace c2d

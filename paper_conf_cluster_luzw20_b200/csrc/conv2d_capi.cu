@@ -1,25 +1,41 @@
-// conv2d_capi.cu -- the C ABI declared in include/conv2d.h: argument validation, launch geometry
-// (band height, F-block), per-K template dispatch, launch on the caller's stream.
+// conv2d_capi.cu -- the C ABI declared in include/conv2d.h: argument validation and per-K dispatch
+// to the launch units (inst_kNN.cu), the Fig. 1a baseline kernel, error strings.
 #include <atomic>
 #include <cstdint>
-#include <cstring>
 #include <mutex>
 
 #include <cuda_runtime.h>
 
 #include "../../include/conv2d.h"
-#include "conv2d_kernels.cuh"
+#include "common.h"
+
+namespace c2d {
+
+std::atomic<int> g_variant{0};
+std::atomic<int> g_min_band{0};
+std::atomic<int> g_mvariant{0};
+
+// ------------------------------------------------------------------------------------------------
+// Baseline: PAPER.md Fig. 1a direct convolution, one thread per output, K*K loads per thread
+// ------------------------------------------------------------------------------------------------
+__global__ void __launch_bounds__(256) k_conv2d_direct(const float *__restrict__ in, int W, const float *__restrict__ filt,
+                                                       int K, float *__restrict__ out, int Ho, int Wo) {
+  const long long idx = static_cast<long long>(blockIdx.x) * blockDim.x + threadIdx.x;
+  if (idx >= static_cast<long long>(Ho) * Wo) return;
+  const int y = static_cast<int>(idx / Wo), x = static_cast<int>(idx % Wo);
+  float s = 0.f;
+  for (int i = 0; i < K; ++i)
+    for (int j = 0; j < K; ++j) s = fmaf(in[static_cast<size_t>(y + i) * W + x + j], __ldg(filt + i * K + j), s);
+  out[idx] = s;
+}
+
+}  // namespace c2d
 
 namespace {
 
 using namespace c2d;
 
 constexpr int kMaxDevices = 64;
-
-struct DevInfo {
-  int num_sms = 0;
-  int smem_optin = 0;
-};
 
 DevInfo g_dev[kMaxDevices];
 std::once_flag g_dev_once[kMaxDevices];
@@ -36,218 +52,10 @@ int current_device_info(DevInfo *out) {
 }
 
 bool aligned4(const void *p) { return (reinterpret_cast<uintptr_t>(p) & 3u) == 0; }
-bool aligned16(const void *p) { return (reinterpret_cast<uintptr_t>(p) & 15u) == 0; }
 
 bool overlap(const void *a, size_t abytes, const void *b, size_t bbytes) {
   const uintptr_t a0 = reinterpret_cast<uintptr_t>(a), b0 = reinterpret_cast<uintptr_t>(b);
   return a0 < b0 + bbytes && b0 < a0 + abytes;
-}
-
-int ceil_div(long long a, long long b) { return static_cast<int>((a + b - 1) / b); }
-
-// Occupancy (CTAs per SM) of a kernel instantiation, cached per instantiation (devices of one box
-// are identical B200s).
-template <typename KernelT>
-int cta_occupancy(KernelT kernel, size_t dyn_smem, std::atomic<int> &cache, int cta_warps = kCtaWarps) {
-  int v = cache.load(std::memory_order_relaxed);
-  if (v > 0) return v;
-  int blocks = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, kernel, cta_warps * kWarp, dyn_smem) != cudaSuccess ||
-      blocks < 1)
-    blocks = 1;
-  cache.store(blocks, std::memory_order_relaxed);
-  return blocks;
-}
-
-// ------------------------------------------------------------------------------------------------
-// single channel
-// ------------------------------------------------------------------------------------------------
-// Variant override for tuning tools (c2d_debug_set_variant; 0 = the tuned default):
-//   1: filter in shared memory, U=1 (4 warps/CTA)     2: shared memory, U=2
-//   3: filter in a __constant__ slot, U=1 (1 warp/CTA) 4: __constant__ slot, U=2
-std::atomic<int> g_variant{0};
-std::atomic<int> g_min_band{0};  // tuning override of the minimum band height (0 = per-K default)
-
-// Constant-bank filter slots, per device: slot K holds the filter of the last call with this K. A
-// call waits (stream-ordered) for the event recorded behind the previous kernel that read the slot
-// before overwriting it, so calls on different streams never see each other's filter; calls with
-// the same K on different streams are serialised by that wait, calls on one stream cost nothing.
-struct ConstRing {
-  std::mutex mu;
-  bool init = false;
-  float *base = nullptr;  // device address of c_filt
-  cudaEvent_t ev[kConstSlots];
-};
-ConstRing g_cring[kMaxDevices];
-
-template <typename LaunchFn>
-int with_const_filter(const float *filt, int K, int KP, cudaStream_t stream, LaunchFn launch) {
-  int dev = 0;
-  if (cudaGetDevice(&dev) != cudaSuccess || dev < 0 || dev >= kMaxDevices) return CONV2D_ECUDA;
-  ConstRing &ring = g_cring[dev];
-  std::lock_guard<std::mutex> lk(ring.mu);
-  if (!ring.init) {
-    void *p = nullptr;
-    if (cudaGetSymbolAddress(&p, c_filt) != cudaSuccess) return CONV2D_ECUDA;
-    ring.base = static_cast<float *>(p);
-    for (int i = 0; i < kConstSlots; ++i)
-      if (cudaEventCreateWithFlags(&ring.ev[i], cudaEventDisableTiming) != cudaSuccess) return CONV2D_ECUDA;
-    ring.init = true;
-  }
-  const int slot = K;
-  if (cudaStreamWaitEvent(stream, ring.ev[slot], 0) != cudaSuccess) return CONV2D_ECUDA;
-  // K rows of K floats -> K rows of KP floats (16-byte aligned rows for LDCU.128)
-  if (cudaMemcpy2DAsync(ring.base + static_cast<size_t>(slot) * kConstSlotFloats, KP * sizeof(float), filt,
-                        K * sizeof(float), K * sizeof(float), K, cudaMemcpyDeviceToDevice, stream) != cudaSuccess)
-    return CONV2D_ECUDA;
-  const int rc = launch();
-  if (rc != CONV2D_OK) return rc;
-  if (cudaEventRecord(ring.ev[slot], stream) != cudaSuccess) return CONV2D_ECUDA;
-  return CONV2D_OK;
-}
-
-bool stream_capturing(cudaStream_t s) {
-  cudaStreamCaptureStatus st = cudaStreamCaptureStatusNone;
-  return cudaStreamIsCapturing(s, &st) == cudaSuccess && st != cudaStreamCaptureStatusNone;
-}
-
-template <int K, int U, int FSRC, int PF = 1, int GUARDS = 0>
-int launch_single_v(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                    const DevInfo &dev, int min_band) {
-  constexpr int CTAW = (FSRC == FSRC_CONST) ? 1 : kCtaWarps;
-  auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS>;
-  static std::atomic<int> occ_cache{0};
-  SingleArgs a;
-  a.in = in;
-  a.filt = filt;
-  a.out = out;
-  a.H = H;
-  a.W = W;
-  a.Ho = H - K + 1;
-  a.Wo = W - K + 1;
-  a.n_cb = ceil_div(a.Wo, 128 * U);
-  a.aligned = (aligned16(in) && (W % 4 == 0)) ? 1 : 0;
-  if (band_h <= 0) {
-    // one full wave of warp tiles: bands = resident warps / column blocks
-    const long long resident_warps =
-        static_cast<long long>(cta_occupancy(kernel, 0, occ_cache, CTAW)) * CTAW * dev.num_sms;
-    const long long bands = resident_warps / a.n_cb > 0 ? resident_warps / a.n_cb : 1;
-    band_h = ceil_div(a.Ho, bands);
-    if (band_h < min_band) band_h = min_band;
-  }
-  if (band_h > a.Ho) band_h = a.Ho;
-  a.band_h = band_h;
-  const int n_bands = ceil_div(a.Ho, band_h);
-  a.n_tiles = a.n_cb * n_bands;
-  const int blocks = ceil_div(a.n_tiles, CTAW);
-  auto go = [&]() {
-    kernel<<<blocks, CTAW * kWarp, 0, stream>>>(a);
-    return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
-  };
-  if constexpr (FSRC == FSRC_CONST) return with_const_filter(filt, K, KCfg<K>::KP, stream, go);
-  return go();
-}
-
-template <int K>
-int launch_single(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                  const DevInfo &dev) {
-  const int mb = g_min_band.load(std::memory_order_relaxed);
-  const int min_band = mb > 0 ? mb : (K - 1 > 4 ? K - 1 : 4);
-  const int v = g_variant.load(std::memory_order_relaxed);
-  // CUDA-graph capture cannot use the event-guarded constant slots: shared-memory filter there
-  const bool constant_ok = !stream_capturing(stream);
-#define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G>(in, H, W, filt, out, stream, band_h, dev, min_band)
-  switch (v) {
-    case 1: return C2D_LS(1, FSRC_SMEM, 1, 0);
-    case 2: return C2D_LS(2, FSRC_SMEM, 1, 0);
-    case 3: if (constant_ok) return C2D_LS(1, FSRC_CONST, 1, 0); break;
-    case 4: if (constant_ok) return C2D_LS(2, FSRC_CONST, 1, 0); break;
-    case 5: if (constant_ok) return C2D_LS(1, FSRC_CONST, 1, 1); break;
-    case 6: if (constant_ok) return C2D_LS(1, FSRC_CONST, 1, 2); break;
-    default: break;
-  }
-  // Tuned on B200 (tools/variants.py, profiles/): two 128-column
-  // chunks per warp while K <= 7 (K = 9 on wide images); above, one chunk with a guarded prologue on
-  // wide images (tall bands) and guarded prologue + epilogue on narrow ones (short bands, where the
-  // wasted FMAs of an unguarded epilogue would be a large fraction).
-  const bool u2 = (K <= 7) || (K <= 9 && W > 3000);
-  if (!constant_ok) return u2 ? C2D_LS(2, FSRC_SMEM, 1, 0) : C2D_LS(1, FSRC_SMEM, 1, 0);
-  if (u2) return C2D_LS(2, FSRC_CONST, 1, 0);
-  if (W >= 4096) return C2D_LS(1, FSRC_CONST, 1, 1);
-  return C2D_LS(1, FSRC_CONST, 1, 2);
-#undef C2D_LS
-}
-
-// ------------------------------------------------------------------------------------------------
-// multi channel
-// ------------------------------------------------------------------------------------------------
-template <int K>
-struct MultiCfg {
-  static constexpr int FB = (K <= 4) ? 8 : (K <= 8 ? 4 : 2);
-};
-
-template <int K, int FB>
-int launch_multi_fb(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
-                    cudaStream_t stream, int band_h, const DevInfo &dev, size_t smem) {
-  auto kernel = k_conv2d_multi<K, FB>;
-  static std::atomic<int> occ_cache{0};
-  static std::atomic<int> smem_set{0};
-  if (smem > 48 * 1024 && smem_set.load() < static_cast<int>(smem)) {
-    if (cudaFuncSetAttribute(kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, dev.smem_optin) != cudaSuccess)
-      return CONV2D_ECUDA;
-    smem_set.store(dev.smem_optin);
-  }
-  MultiArgs a;
-  a.in = in;
-  a.filt = filt;
-  a.out = out;
-  a.N = N;
-  a.C = C;
-  a.H = H;
-  a.W = W;
-  a.F = F;
-  a.Ho = H - K + 1;
-  a.Wo = W - K + 1;
-  a.n_cb = ceil_div(a.Wo, 128);
-  a.n_fb = ceil_div(F, FB);
-  a.aligned = (aligned16(in) && (W % 4 == 0)) ? 1 : 0;
-  if (band_h <= 0) {
-    // occupancy of this instantiation with this smem size (the cache holds the value for the
-    // first smem size seen; good enough for choosing a band height)
-    const long long resident_warps =
-        static_cast<long long>(cta_occupancy(kernel, smem, occ_cache)) * kCtaWarps * dev.num_sms;
-    const long long groups = static_cast<long long>(N) * a.n_fb * a.n_cb;
-    long long bands = resident_warps / groups;
-    if (bands < 1) bands = 1;
-    band_h = ceil_div(a.Ho, bands);
-    const int min_band = 4;
-    if (band_h < min_band) band_h = min_band;
-  }
-  if (band_h > a.Ho) band_h = a.Ho;
-  a.band_h = band_h;
-  int n_bands = ceil_div(a.Ho, band_h);
-  // all 4 warps of a CTA must share (n, F-block): pad the tiles per (n, F-block) to a multiple of 4
-  while ((static_cast<long long>(a.n_cb) * n_bands) % kCtaWarps) ++n_bands;
-  a.n_bands = n_bands;
-  a.n_tiles = static_cast<long long>(N) * a.n_fb * n_bands * a.n_cb;
-  const long long blocks = (a.n_tiles + kCtaWarps - 1) / kCtaWarps;
-  if (blocks > 0x7fffffffLL) return CONV2D_ESHAPE;
-  kernel<<<static_cast<unsigned>(blocks), kCtaWarps * kWarp, smem, stream>>>(a);
-  return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
-}
-
-template <int K>
-int launch_multi(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
-                 cudaStream_t stream, int band_h, const DevInfo &dev) {
-  constexpr int FB = MultiCfg<K>::FB;
-  constexpr int KP = KCfg<K>::KP;
-  const size_t smem = static_cast<size_t>(C) * K * FB * KP * sizeof(float);
-  if (smem <= static_cast<size_t>(dev.smem_optin))
-    return launch_multi_fb<K, FB>(in, N, C, H, W, filt, F, out, stream, band_h, dev, smem);
-  const size_t smem1 = static_cast<size_t>(C) * K * KP * sizeof(float);
-  if (smem1 <= static_cast<size_t>(dev.smem_optin))
-    return launch_multi_fb<K, 1>(in, N, C, H, W, filt, F, out, stream, band_h, dev, smem1);
-  return CONV2D_ESHAPE;
 }
 
 #define C2D_K_SWITCH(K, CALL) \
@@ -293,7 +101,7 @@ int conv2d_single_ex(const float *in, int H, int W, const float *filt, int K, fl
   DevInfo dev;
   if (current_device_info(&dev)) return CONV2D_ECUDA;
   cudaStream_t s = static_cast<cudaStream_t>(stream);
-#define C2D_CALL_SINGLE(KK) launch_single<KK>(in, H, W, filt, out, s, band_h, dev)
+#define C2D_CALL_SINGLE(KK) single_entry<KK>(in, H, W, filt, out, s, band_h, dev)
   C2D_K_SWITCH(K, C2D_CALL_SINGLE)
 #undef C2D_CALL_SINGLE
 }
@@ -319,7 +127,7 @@ int conv2d_multi_ex(const float *in, int N, int C, int H, int W, const float *fi
   DevInfo dev;
   if (current_device_info(&dev)) return CONV2D_ECUDA;
   cudaStream_t s = static_cast<cudaStream_t>(stream);
-#define C2D_CALL_MULTI(KK) launch_multi<KK>(in, N, C, H, W, filt, F, out, s, band_h, dev)
+#define C2D_CALL_MULTI(KK) multi_entry<KK>(in, N, C, H, W, filt, F, out, s, band_h, dev)
   C2D_K_SWITCH(K, C2D_CALL_MULTI)
 #undef C2D_CALL_MULTI
 }
@@ -365,6 +173,13 @@ int conv2d_version(void) { return 100; }
 // Not part of include/conv2d.h: selects a kernel variant for tuning tools (0 = default).
 int c2d_debug_set_variant(int v) {
   const int old = g_variant.exchange(v);
+  return old;
+}
+
+// Not part of include/conv2d.h: multi-channel variant for tuning tools (0 = default; 1/2 constant
+// filters wide/narrow segments; 3/4 shared-memory filters wide/narrow; 9 = round-1 kernel).
+int c2d_debug_set_multi_variant(int v) {
+  const int old = g_mvariant.exchange(v);
   return old;
 }
 

@@ -29,8 +29,8 @@
 //     accumulators; each thread also carries FB filters, so one window feeds FB*K*K*4 FMAs.
 //   * a6 Output store: slot 0 is complete after each row -> one coalesced store per lane; rows whose
 //     pitch breaks 16-byte alignment are realigned with warp shuffles (static per-shift variants).
-// Edge tiles (ragged right edge) and misaligned tensors take the same code with guarded scalar
-// loads/stores (SAFE=true).
+// Edge tiles (ragged right edge: clamped vector loads, masked stores) and misaligned tensors (scalar
+// loads/stores) take the same code with SAFE=true.
 #pragma once
 
 #include <cstdint>
@@ -74,45 +74,63 @@ struct RowBuf {
   float e[4];
 };
 
-// rowp points at input column 0 of the row. SAFE: guarded scalar loads (ragged edge / misaligned).
-template <int K, int U, bool SAFE>
-__device__ __forceinline__ void load_row(RowBuf<K, U> &b, const float *__restrict__ rowp, int x0, int W,
-                                         int lane) {
+// One row segment of a warp tile. The warp is split into 32/SEG segments of SEG lanes; segment lane
+// sl holds columns x0 + 4*SEG*u + 4*sl + {0..3} of chunk u < U, plus (lanes sl < NE) one quad of the
+// K-1 halo columns right of the segment's span. rowp points at input column 0 of the row.
+//   SAFE == false: the whole span + halo is inside the row and 16-byte aligned: LDG.128 per lane,
+//                  and every lane loads a halo quad (lanes >= NE re-read a duplicate: branch-free).
+//   SAFE == true : ragged right edge or misaligned rows. Aligned rows (W % 4 == 0, 16-byte base):
+//                  the quad address is clamped to the last quad of the row -- quads are either fully
+//                  inside or fully outside the row, and a valid output only reads inside quads, so
+//                  the clamped (garbage) values only reach outputs >= Wo, which are never stored.
+//                  Misaligned rows: guarded scalar loads.
+template <int K, int U, int SEG, bool SAFE>
+__device__ __forceinline__ void load_row_g(RowBuf<K, U> &b, const float *__restrict__ rowp, int x0, int W, int sl,
+                                           bool aligned) {
+  constexpr int NE = KCfg<K>::NE;
 #pragma unroll
   for (int u = 0; u < U; ++u) {
-    const int x = x0 + 128 * u + 4 * lane;
-    if (!SAFE) {
-      const float4 v = ldg4(rowp + x);
+    const int x = x0 + 4 * SEG * u + 4 * sl;
+    if (!SAFE || aligned) {
+      const float4 v = ldg4(rowp + (SAFE ? min(x, W - 4) : x));
       b.a[u][0] = v.x; b.a[u][1] = v.y; b.a[u][2] = v.z; b.a[u][3] = v.w;
     } else {
 #pragma unroll
       for (int t = 0; t < 4; ++t) b.a[u][t] = (x + t < W) ? __ldg(rowp + x + t) : 0.f;
     }
   }
-  if constexpr (KCfg<K>::NE == 0) {
+  const int xe = x0 + 4 * SEG * U + 4 * (sl % (NE > 0 ? NE : 1));
+  if constexpr (NE == 0) {
 #pragma unroll
     for (int t = 0; t < 4; ++t) b.e[t] = 0.f;
-  } else if constexpr (!SAFE) {
-    // fast tiles guarantee x0 + 128U + 4*NE <= W: every lane loads (lanes >= NE re-read lane
-    // (l mod NE)'s quad, same sectors), no branch
-    const float4 v = ldg4(rowp + x0 + 128 * U + 4 * (lane % KCfg<K>::NE));
-    b.e[0] = v.x; b.e[1] = v.y; b.e[2] = v.z; b.e[3] = v.w;
   } else {
+    if (!SAFE || aligned) {
+      const float4 v = ldg4(rowp + (SAFE ? min(xe, W - 4) : xe));
+      b.e[0] = v.x; b.e[1] = v.y; b.e[2] = v.z; b.e[3] = v.w;
+    } else {
 #pragma unroll
-    for (int t = 0; t < 4; ++t) b.e[t] = 0.f;
-    if (lane < KCfg<K>::NE) {
-      const int x = x0 + 128 * U + 4 * lane;
-#pragma unroll
-      for (int t = 0; t < 4; ++t) b.e[t] = (x + t < W) ? __ldg(rowp + x + t) : 0.f;
+      for (int t = 0; t < 4; ++t) b.e[t] = (sl < NE && xe + t < W) ? __ldg(rowp + xe + t) : 0.f;
     }
   }
 }
 
+template <int K, int U, bool SAFE>
+__device__ __forceinline__ void load_row(RowBuf<K, U> &b, const float *__restrict__ rowp, int x0, int W, int lane,
+                                         bool aligned) {
+  load_row_g<K, U, kWarp, SAFE>(b, rowp, x0, W, lane, aligned);
+}
+
 // ------------------------------------------------------------------------------------------------
-// a2: column reuse -- assemble every chunk's window w[u][0..WN) = in[x0+128u+4l .. +WN)
+// a2: column reuse -- assemble every chunk's window w[u][0..WN) = in[x0+4*SEG*u+4*sl .. +WN)
 // ------------------------------------------------------------------------------------------------
-template <int K, int U>
-__device__ __forceinline__ void build_windows(const RowBuf<K, U> &b, float (&w)[U][KCfg<K>::WN], int lane) {
+// Halo element m (m = 4..K+2) of segment lane sl lives in register m%4 of segment lane sl + m/4.
+// The SUPPLYING lane picks, with a static register index, its own register or -- if it is one of the
+// first m/4 lanes, whose receivers wrap past the segment's last lane -- the next chunk's (or the halo
+// quad's) register; one SEL + one SHFL.IDX (source lane inside the segment) per (m, chunk).
+template <int K, int U, int SEG>
+__device__ __forceinline__ void build_windows_g(const RowBuf<K, U> &b, float (&w)[U][KCfg<K>::WN], int lane) {
+  const int sl = lane & (SEG - 1);
+  const int base = lane & ~(SEG - 1);
 #pragma unroll
   for (int u = 0; u < U; ++u) {
 #pragma unroll
@@ -122,16 +140,19 @@ __device__ __forceinline__ void build_windows(const RowBuf<K, U> &b, float (&w)[
   for (int m = 4; m < KCfg<K>::WN; ++m) {
     const int d = m >> 2;  // source lane offset (static)
     const int r = m & 3;   // source register (static)
-    const int src = (lane + d) & (kWarp - 1);
+    const int src = base | ((sl + d) & (SEG - 1));
 #pragma unroll
     for (int u = 0; u < U; ++u) {
-      // Lanes s < d supply the NEXT chunk's register r (for receivers that wrap past lane 31);
-      // lanes s >= d supply their own register r. Static register index, lane-dependent select.
       const float nxt = (u + 1 < U) ? b.a[(u + 1 < U) ? u + 1 : 0][r] : b.e[r];
-      const float sup = (lane < d) ? nxt : b.a[u][r];
+      const float sup = (sl < d) ? nxt : b.a[u][r];
       w[u][m] = __shfl_sync(kFull, sup, src);
     }
   }
+}
+
+template <int K, int U>
+__device__ __forceinline__ void build_windows(const RowBuf<K, U> &b, float (&w)[U][KCfg<K>::WN], int lane) {
+  build_windows_g<K, U, kWarp>(b, w, lane);
 }
 
 // ------------------------------------------------------------------------------------------------
@@ -152,8 +173,9 @@ constexpr int FSRC_SMEM = 0;
 constexpr int FSRC_CONST = 1;
 
 constexpr int kConstSlotFloats = 256;  // >= 15 rows x 16 (padded) floats
-constexpr int kConstSlots = 16;        // slot K for K = 1..15 (16 KiB of the 64 KiB constant bank)
-__constant__ __align__(16) float c_filt[kConstSlots * kConstSlotFloats];
+// One slot per translation unit: every K is compiled in its own unit (csrc/inst_kNN.cu) and so in its
+// own module with its own constant bank; slot "K" of the design is this array in unit K.
+__constant__ __align__(16) float c_filt[kConstSlotFloats];
 
 __device__ __forceinline__ void lds4_at(unsigned saddr, float &a, float &b, float &c, float &d) {
   asm volatile("ld.shared.v4.f32 {%0, %1, %2, %3}, [%4];" : "=f"(a), "=f"(b), "=f"(c), "=f"(d) : "r"(saddr));
@@ -162,7 +184,7 @@ __device__ __forceinline__ void lds4_at(unsigned saddr, float &a, float &b, floa
 template <int K, int FSRC>
 struct FilterSrc {
   unsigned sbase;      // FSRC_SMEM: shared-window address of row 0
-  const float *cbase;  // FSRC_CONST: slot K of c_filt (compile-time address, rows of KP floats)
+  const float *cbase;  // FSRC_CONST: c_filt of this unit (compile-time address, rows of KP floats)
 
   __device__ __forceinline__ void row(float (&fr)[KCfg<K>::KP], int i) const {
     constexpr int KP = KCfg<K>::KP;
@@ -312,16 +334,16 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc
 #pragma unroll
       for (int v = 0; v < 4; ++v) acc[q][u][v] = 0.f;
   RowBuf<K, U> n1, n2;  // rows r+1 (and r+2 when PF == 2) in flight
-  load_row<K, U, SAFE>(n1, in_row(a, ob), x0, a.W, lane);
-  if (PF == 2) load_row<K, U, SAFE>(n2, in_row(a, min(ob + 1, rlast)), x0, a.W, lane);
+  load_row<K, U, SAFE>(n1, in_row(a, ob), x0, a.W, lane, a.aligned);
+  if (PF == 2) load_row<K, U, SAFE>(n2, in_row(a, min(ob + 1, rlast)), x0, a.W, lane, a.aligned);
   // advance the in-flight rows: returns row r, issues the load of row r+PF (index clamped)
   auto next_row = [&](int r) {
     const RowBuf<K, U> cur = n1;
     if constexpr (PF == 2) {
       n1 = n2;
-      load_row<K, U, SAFE>(n2, in_row(a, min(r + 2, rlast)), x0, a.W, lane);
+      load_row<K, U, SAFE>(n2, in_row(a, min(r + 2, rlast)), x0, a.W, lane, a.aligned);
     } else {
-      load_row<K, U, SAFE>(n1, in_row(a, min(r + 1, rlast)), x0, a.W, lane);
+      load_row<K, U, SAFE>(n1, in_row(a, min(r + 1, rlast)), x0, a.W, lane, a.aligned);
     }
     return cur;
   };
@@ -368,7 +390,7 @@ __global__ void __launch_bounds__(CTAW *kWarp) k_conv2d_single(const SingleArgs 
   __shared__ __align__(16) float sf[(FSRC == FSRC_SMEM) ? K * KP : 4];
   FilterSrc<K, FSRC> fs;
   if constexpr (FSRC == FSRC_CONST) {
-    fs.cbase = c_filt + K * kConstSlotFloats;
+    fs.cbase = c_filt;
   } else {
     for (int t = threadIdx.x; t < K * KP; t += blockDim.x) {
       const int i = t / KP, j = t % KP;
@@ -457,7 +479,7 @@ __device__ __forceinline__ void multi_tile(const MultiArgs &a, const float *__re
       for (int v = 0; v < 4; ++v) acc[q][fb][v] = 0.f;
 
   RowBuf<K, 1> nxt;
-  load_row<K, 1, SAFE>(nxt, img + static_cast<size_t>(ob) * a.W, x0, a.W, lane);
+  load_row<K, 1, SAFE>(nxt, img + static_cast<size_t>(ob) * a.W, x0, a.W, lane, a.aligned);
   for (int r = ob; r < rend; ++r) {
     const int done = r - ob;
     const int qmin = (done < K - 1) ? (K - 1 - done) : 0;
@@ -468,7 +490,7 @@ __device__ __forceinline__ void multi_tile(const MultiArgs &a, const float *__re
         int rn = r, cn = c + 1;
         if (cn == C) { cn = 0; ++rn; }
         if (rn < rend)
-          load_row<K, 1, SAFE>(nxt, img + cn * plane + static_cast<size_t>(rn) * a.W, x0, a.W, lane);
+          load_row<K, 1, SAFE>(nxt, img + cn * plane + static_cast<size_t>(rn) * a.W, x0, a.W, lane, a.aligned);
       }
       float w[1][KCfg<K>::WN];
       build_windows<K, 1>(cur, w, lane);
@@ -529,20 +551,6 @@ __global__ void __launch_bounds__(kCtaWarps *kWarp) k_conv2d_multi(const MultiAr
     multi_tile<K, FB, false>(a, smem, n, f0, x0, ob, oe, lane);
   else
     multi_tile<K, FB, true>(a, smem, n, f0, x0, ob, oe, lane);
-}
-
-// ------------------------------------------------------------------------------------------------
-// Baseline: PAPER.md Fig. 1a direct convolution, one thread per output, K*K loads per thread
-// ------------------------------------------------------------------------------------------------
-__global__ void __launch_bounds__(256) k_conv2d_direct(const float *__restrict__ in, int W, const float *__restrict__ filt,
-                                                       int K, float *__restrict__ out, int Ho, int Wo) {
-  const long long idx = static_cast<long long>(blockIdx.x) * blockDim.x + threadIdx.x;
-  if (idx >= static_cast<long long>(Ho) * Wo) return;
-  const int y = static_cast<int>(idx / Wo), x = static_cast<int>(idx % Wo);
-  float s = 0.f;
-  for (int i = 0; i < K; ++i)
-    for (int j = 0; j < K; ++j) s = fmaf(in[static_cast<size_t>(y + i) * W + x + j], __ldg(filt + i * K + j), s);
-  out[idx] = s;
 }
 
 }  // namespace c2d

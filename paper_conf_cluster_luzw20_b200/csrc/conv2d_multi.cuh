@@ -1,0 +1,220 @@
+// conv2d_multi.cuh -- multi-channel kernel (N images x C channels x F filters of K x K), sm_100a.
+//
+// The single-channel design (conv2d_kernels.cuh) extended along the two new axes of PAPER.md's
+// multi-channel experiment (Table I):
+//   * a5 channel reduction: for every input row r the C channel rows stream through the same K-slot
+//     accumulator ring (the first channel also shifts the ring), so each output sums its C*K*K terms
+//     in (filter row, channel, filter column) order, band-independent;
+//   * FB filters per warp: one assembled window (column reuse) feeds K slots x FB filters x 4 x K FMAs;
+//   * SEG-lane segments: a warp is split into 32/SEG segments of SEG lanes (4*SEG columns each) that
+//     work on different images n with identical control flow, so narrow images (e.g. the 54-column
+//     outputs of 56x56 layers) do not leave most lanes idle. The column-reuse shuffles wrap inside a
+//     segment (shfl.idx with a segment-local source lane);
+//   * U chunks of 4*SEG columns per segment share every filter-row fetch (more FMAs per LDS);
+//   * filters: the CTA's F-block staged in shared memory (4 warps per CTA share it), broadcast LDS.128.
+//     (A __constant__ filter bank read through uniform registers -- the single-channel choice -- does
+//     not work here: warps on one SM use different F-blocks, the working set overflows the constant
+//     cache and LDCU latency serialises the warp; measured 3 vs 24 TFLOP/s on configs[3].)
+// Alg. 2's first/last K-1 rows of a band (cases 1 and 3) are guarded per slot (GUARDS=2) when bands
+// are short, or run the full body (GUARDS=0) when bands are tall.
+#pragma once
+
+#include <type_traits>
+
+#include "conv2d_kernels.cuh"
+
+namespace c2d {
+
+struct Multi2Args {
+  const float *in;
+  const float *filt;  // F x C x K x K in global memory
+  float *out;
+  int N, C, H, W, F, Ho, Wo;
+  int band_h, n_cb, n_bands, n_fb, n_groups;
+  long long n_tiles;
+  int aligned;
+};
+
+// filter row (fb, c, i) of the CTA's F-block, staged in shared memory as [c][i][fb][KP]
+template <int K, int FB>
+struct MultiFilter {
+  unsigned sbase;
+
+  __device__ __forceinline__ void row(float (&fr)[KCfg<K>::KP], int fb, int c, int i) const {
+    constexpr int KP = KCfg<K>::KP;
+#pragma unroll
+    for (int c4 = 0; c4 < KP / 4; ++c4)
+      lds4_at(sbase + static_cast<unsigned>((((c * K + i) * FB + fb) * KP + 4 * c4) * 4), fr[4 * c4],
+              fr[4 * c4 + 1], fr[4 * c4 + 2], fr[4 * c4 + 3]);
+  }
+};
+
+// a3 + a5: one (row, channel) into the ring of FB filters x U chunks
+template <int K, int FB, int U, bool SHIFT, bool GUARD>
+__device__ __forceinline__ void row_step_multi(float (&acc)[K][FB][U][4], const float (&w)[U][KCfg<K>::WN],
+                                               const MultiFilter<K, FB> &mf, int c, int qmin, int qmax) {
+#pragma unroll
+  for (int q = 0; q < K; ++q) {
+    if (!GUARD || (q >= qmin && q < qmax)) {
+#pragma unroll
+      for (int fb = 0; fb < FB; ++fb) {
+        float fr[KCfg<K>::KP];
+        mf.row(fr, fb, c, K - 1 - q);
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+#pragma unroll
+          for (int v = 0; v < 4; ++v) {
+            float s;
+            if (SHIFT)
+              s = (q + 1 < K) ? acc[(q + 1 < K) ? q + 1 : 0][fb][u][v] : 0.f;
+            else
+              s = acc[q][fb][u][v];
+#pragma unroll
+            for (int j = 0; j < K; ++j) s = fmaf(w[u][v + j], fr[j], s);
+            acc[q][fb][u][v] = s;
+          }
+        }
+      }
+    }
+  }
+}
+
+template <int K, int FB, int U, int SEG, int GUARDS, int PF, bool SAFE>
+__device__ __forceinline__ void multi_tile2(const Multi2Args &a, const MultiFilter<K, FB> &mf, int n,
+                                            bool seg_active, int f0, int x0, int ob, int oe, int lane) {
+  const int sl = lane & (SEG - 1);
+  const int C = a.C;
+  const int rend = oe + K - 1;
+  const int rlast = rend - 1;
+  const size_t plane = static_cast<size_t>(a.H) * a.W;
+  const float *__restrict__ img = a.in + static_cast<size_t>(n) * C * plane;
+  float acc[K][FB][U][4];
+#pragma unroll
+  for (int q = 0; q < K; ++q)
+#pragma unroll
+    for (int fb = 0; fb < FB; ++fb)
+#pragma unroll
+      for (int u = 0; u < U; ++u)
+#pragma unroll
+        for (int v = 0; v < 4; ++v) acc[q][fb][u][v] = 0.f;
+
+  // the (row, channel) stream: (r, c) -> (r, c+1) -> ... -> (r+1, 0); PF = 1 or 2 entries in flight
+  auto row_ptr = [&](int r, int c) { return img + c * plane + static_cast<size_t>(r) * a.W; };
+  RowBuf<K, U> n1, n2;
+  int pr = ob, pc = 0;  // (row, channel) of the next load to issue
+  auto advance = [&]() {
+    if (++pc == C) {
+      pc = 0;
+      pr = min(pr + 1, rlast);
+    }
+  };
+  load_row_g<K, U, SEG, SAFE>(n1, row_ptr(pr, pc), x0, a.W, sl, a.aligned);
+  advance();
+  if constexpr (PF == 2) {
+    load_row_g<K, U, SEG, SAFE>(n2, row_ptr(pr, pc), x0, a.W, sl, a.aligned);
+    advance();
+  }
+  auto stream_row = [&](int r, int qmin, int qmax, auto guard_tag) {
+    constexpr bool G = decltype(guard_tag)::value;
+    for (int c = 0; c < C; ++c) {
+      const RowBuf<K, U> cur = n1;
+      if constexpr (PF == 2) {
+        n1 = n2;
+        load_row_g<K, U, SEG, SAFE>(n2, row_ptr(pr, pc), x0, a.W, sl, a.aligned);
+      } else {
+        load_row_g<K, U, SEG, SAFE>(n1, row_ptr(pr, pc), x0, a.W, sl, a.aligned);
+      }
+      advance();
+      float w[U][KCfg<K>::WN];
+      build_windows_g<K, U, SEG>(cur, w, lane);
+      if (c == 0)
+        row_step_multi<K, FB, U, true, G>(acc, w, mf, c, qmin, qmax);
+      else
+        row_step_multi<K, FB, U, false, G>(acc, w, mf, c, qmin, qmax);
+    }
+  };
+  auto store_slot0 = [&](int o) {
+#pragma unroll
+    for (int fb = 0; fb < FB; ++fb) {
+      const int f = f0 + fb;
+      if (f < a.F) {
+        float *orow = a.out + ((static_cast<size_t>(n) * a.F + f) * a.Ho + o) * a.Wo;
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+          const int xb = x0 + 4 * SEG * u;
+          if constexpr (SEG == kWarp && !SAFE) {
+            store_chunk(orow + xb, acc[0][fb][u], lane);
+          } else if (seg_active) {
+#pragma unroll
+            for (int t = 0; t < 4; ++t) {
+              const int x = xb + 4 * sl + t;
+              if (x < a.Wo) __stcs(orow + x, acc[0][fb][u][t]);
+            }
+          }
+        }
+      }
+    }
+  };
+  int r = ob;
+  if constexpr (GUARDS == 0) {
+    for (; r < rend; ++r) {
+      stream_row(r, 0, K, std::false_type{});
+      if (r >= ob + K - 1) store_slot0(r - K + 1);
+    }
+  } else {
+    for (; r < min(ob + K - 1, oe); ++r) stream_row(r, K - 1 - (r - ob), K, std::true_type{});
+    for (; r < oe; ++r) {
+      stream_row(r, 0, K, std::false_type{});
+      store_slot0(r - K + 1);
+    }
+    for (; r < rend; ++r) {
+      stream_row(r, max(0, K - 1 - (r - ob)), oe + K - 1 - r, std::true_type{});
+      if (r >= ob + K - 1) store_slot0(r - K + 1);
+    }
+  }
+}
+
+// Tiles are ordered ((group * n_fb + fblk) * n_bands + band) * n_cb + cb; the host pads n_bands so that
+// the CTA's warps share (group, fblk): the CTA stages that F-block's C*K*FB*KP floats once.
+template <int K, int FB, int U, int SEG, int GUARDS, int PF>
+__global__ void __launch_bounds__(kCtaWarps *kWarp) k_conv2d_multi2(const Multi2Args a) {
+  constexpr int KP = KCfg<K>::KP;
+  extern __shared__ __align__(16) float smem[];
+  const long long tile0 = static_cast<long long>(blockIdx.x) * kCtaWarps;
+  const long long per_fb = static_cast<long long>(a.n_cb) * a.n_bands;
+  const int fblk = static_cast<int>((tile0 / per_fb) % a.n_fb);
+  const int f0 = fblk * FB;
+  const int total = a.C * K * FB * KP;
+  for (int t = threadIdx.x; t < total; t += blockDim.x) {
+    const int j = t % KP;
+    const int fb = (t / KP) % FB;
+    const int i = (t / (KP * FB)) % K;
+    const int c = t / (KP * FB * K);
+    const int f = f0 + fb;
+    smem[t] = (j < K && f < a.F) ? a.filt[((static_cast<size_t>(f) * a.C + c) * K + i) * K + j] : 0.f;
+  }
+  __syncthreads();
+  MultiFilter<K, FB> mf;
+  mf.sbase = static_cast<unsigned>(__cvta_generic_to_shared(smem));
+  const int lane = threadIdx.x & (kWarp - 1);
+  const long long tile = tile0 + (threadIdx.x >> 5);
+  if (tile >= a.n_tiles) return;
+  const int cb = static_cast<int>(tile % a.n_cb);
+  const int band = static_cast<int>((tile / a.n_cb) % a.n_bands);
+  const int group = static_cast<int>(tile / (per_fb * a.n_fb));
+  const int ob = band * a.band_h;
+  if (ob >= a.Ho) return;
+  const int oe = min(ob + a.band_h, a.Ho);
+  const int x0 = cb * 4 * SEG * U;
+  constexpr int SEGS = kWarp / SEG;
+  const int n_raw = group * SEGS + lane / SEG;
+  const bool seg_active = n_raw < a.N;
+  const int n = seg_active ? n_raw : a.N - 1;  // idle segments recompute the last image, never store
+  const bool fast = a.aligned && (x0 + 4 * SEG * U + 4 * KCfg<K>::NE <= a.W);  // uniform per warp
+  if (fast)
+    multi_tile2<K, FB, U, SEG, GUARDS, PF, false>(a, mf, n, seg_active, f0, x0, ob, oe, lane);
+  else
+    multi_tile2<K, FB, U, SEG, GUARDS, PF, true>(a, mf, n, seg_active, f0, x0, ob, oe, lane);
+}
+
+}  // namespace c2d

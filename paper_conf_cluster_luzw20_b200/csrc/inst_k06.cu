@@ -1,0 +1,8 @@
+// inst_k06.cu -- kernels and launch code for K = 6 (one K per unit: own constant bank, parallel build)
+#include "launch.cuh"
+
+namespace c2d {
+template int single_entry<6>(const float *, int, int, const float *, float *, cudaStream_t, int, const DevInfo &);
+template int multi_entry<6>(const float *, int, int, int, int, const float *, int, float *, cudaStream_t, int,
+                             const DevInfo &);
+}  // namespace c2d

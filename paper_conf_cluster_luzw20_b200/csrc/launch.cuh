@@ -1,0 +1,323 @@
+// launch.cuh -- host-side launch code of the kernels for one K (included once per translation unit
+// csrc/inst_kNN.cu): launch geometry (band height, F-block, segments), filter staging (constant slot
+// or shared memory), kernel-variant selection. State (constant-slot events, occupancy caches) has
+// internal linkage: one copy per unit, i.e. per K, matching the per-unit constant banks.
+#pragma once
+
+#include <atomic>
+#include <cstdint>
+#include <mutex>
+
+#include <cuda_runtime.h>
+
+#include "common.h"
+#include "conv2d_kernels.cuh"
+#include "conv2d_multi.cuh"
+
+namespace {
+
+using namespace c2d;
+
+constexpr int kMaxDevices = 64;
+
+bool aligned16(const void *p) { return (reinterpret_cast<uintptr_t>(p) & 15u) == 0; }
+
+int ceil_div(long long a, long long b) { return static_cast<int>((a + b - 1) / b); }
+
+// Occupancy (CTAs per SM) of a kernel instantiation, cached per instantiation (devices of one box
+// are identical B200s).
+template <typename KernelT>
+int cta_occupancy(KernelT kernel, size_t dyn_smem, std::atomic<int> &cache, int cta_warps = kCtaWarps) {
+  int v = cache.load(std::memory_order_relaxed);
+  if (v > 0) return v;
+  int blocks = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, kernel, cta_warps * kWarp, dyn_smem) != cudaSuccess ||
+      blocks < 1)
+    blocks = 1;
+  cache.store(blocks, std::memory_order_relaxed);
+  return blocks;
+}
+
+// ------------------------------------------------------------------------------------------------
+// single channel
+// ------------------------------------------------------------------------------------------------
+// Variant override for tuning tools (c2d_debug_set_variant; 0 = the tuned default):
+//   1: filter in shared memory, U=1 (4 warps/CTA)     2: shared memory, U=2
+//   3: filter in a __constant__ slot, U=1 (1 warp/CTA) 4: __constant__ slot, U=2
+
+// Constant-bank filter slot of this unit (this K), per device: it holds the filter of the last call
+// with this K. A call waits (stream-ordered) for the event recorded behind the previous kernel that
+// read the slot before overwriting it, so calls on different streams never see each other's filter;
+// calls with the same K on different streams are serialised by that wait, calls on one stream cost
+// nothing.
+struct ConstRing {
+  std::mutex mu;
+  bool init = false;
+  float *base = nullptr;  // device address of c_filt
+  cudaEvent_t ev;
+};
+ConstRing g_cring[kMaxDevices];
+
+template <typename LaunchFn>
+int with_const_filter(const float *filt, int K, int KP, cudaStream_t stream, LaunchFn launch) {
+  int dev = 0;
+  if (cudaGetDevice(&dev) != cudaSuccess || dev < 0 || dev >= kMaxDevices) return CONV2D_ECUDA;
+  ConstRing &ring = g_cring[dev];
+  std::lock_guard<std::mutex> lk(ring.mu);
+  if (!ring.init) {
+    void *p = nullptr;
+    if (cudaGetSymbolAddress(&p, c_filt) != cudaSuccess) return CONV2D_ECUDA;
+    ring.base = static_cast<float *>(p);
+    if (cudaEventCreateWithFlags(&ring.ev, cudaEventDisableTiming) != cudaSuccess) return CONV2D_ECUDA;
+    ring.init = true;
+  }
+  if (cudaStreamWaitEvent(stream, ring.ev, 0) != cudaSuccess) return CONV2D_ECUDA;
+  // K rows of K floats -> K rows of KP floats (16-byte aligned rows for LDCU.128)
+  if (cudaMemcpy2DAsync(ring.base, KP * sizeof(float), filt, K * sizeof(float), K * sizeof(float), K,
+                        cudaMemcpyDeviceToDevice, stream) != cudaSuccess)
+    return CONV2D_ECUDA;
+  const int rc = launch();
+  if (rc != CONV2D_OK) return rc;
+  if (cudaEventRecord(ring.ev, stream) != cudaSuccess) return CONV2D_ECUDA;
+  return CONV2D_OK;
+}
+
+bool stream_capturing(cudaStream_t s) {
+  cudaStreamCaptureStatus st = cudaStreamCaptureStatusNone;
+  return cudaStreamIsCapturing(s, &st) == cudaSuccess && st != cudaStreamCaptureStatusNone;
+}
+
+template <int K, int U, int FSRC, int PF = 1, int GUARDS = 0>
+int launch_single_v(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
+                    const DevInfo &dev, int min_band) {
+  constexpr int CTAW = (FSRC == FSRC_CONST) ? 1 : kCtaWarps;
+  auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS>;
+  static std::atomic<int> occ_cache{0};
+  SingleArgs a;
+  a.in = in;
+  a.filt = filt;
+  a.out = out;
+  a.H = H;
+  a.W = W;
+  a.Ho = H - K + 1;
+  a.Wo = W - K + 1;
+  a.n_cb = ceil_div(a.Wo, 128 * U);
+  a.aligned = (aligned16(in) && (W % 4 == 0)) ? 1 : 0;
+  if (band_h <= 0) {
+    // one full wave of warp tiles: bands = resident warps / column blocks
+    const long long resident_warps =
+        static_cast<long long>(cta_occupancy(kernel, 0, occ_cache, CTAW)) * CTAW * dev.num_sms;
+    const long long bands = resident_warps / a.n_cb > 0 ? resident_warps / a.n_cb : 1;
+    band_h = ceil_div(a.Ho, bands);
+    if (band_h < min_band) band_h = min_band;
+  }
+  if (band_h > a.Ho) band_h = a.Ho;
+  a.band_h = band_h;
+  const int n_bands = ceil_div(a.Ho, band_h);
+  a.n_tiles = a.n_cb * n_bands;
+  const int blocks = ceil_div(a.n_tiles, CTAW);
+  auto go = [&]() {
+    kernel<<<blocks, CTAW * kWarp, 0, stream>>>(a);
+    return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
+  };
+  if constexpr (FSRC == FSRC_CONST) return with_const_filter(filt, K, KCfg<K>::KP, stream, go);
+  return go();
+}
+
+template <int K>
+int launch_single(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
+                  const DevInfo &dev) {
+  const int mb = g_min_band.load(std::memory_order_relaxed);
+  const int min_band = mb > 0 ? mb : (K - 1 > 4 ? K - 1 : 4);
+  const int v = g_variant.load(std::memory_order_relaxed);
+  // CUDA-graph capture cannot use the event-guarded constant slots: shared-memory filter there
+  const bool constant_ok = !stream_capturing(stream);
+#define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G>(in, H, W, filt, out, stream, band_h, dev, min_band)
+  switch (v) {
+    case 1: return C2D_LS(1, FSRC_SMEM, 1, 0);
+    case 2: return C2D_LS(2, FSRC_SMEM, 1, 0);
+    case 3: if (constant_ok) return C2D_LS(1, FSRC_CONST, 1, 0); break;
+    case 4: if (constant_ok) return C2D_LS(2, FSRC_CONST, 1, 0); break;
+    case 5: if (constant_ok) return C2D_LS(1, FSRC_CONST, 1, 1); break;
+    case 6: if (constant_ok) return C2D_LS(1, FSRC_CONST, 1, 2); break;
+    default: break;
+  }
+  // Tuned on B200 (tools/variants.py, profiles/): two 128-column
+  // chunks per warp while K <= 7 (K = 9 on wide images); above, one chunk with a guarded prologue on
+  // wide images (tall bands) and guarded prologue + epilogue on narrow ones (short bands, where the
+  // wasted FMAs of an unguarded epilogue would be a large fraction).
+  const bool u2 = (K <= 7) || (K <= 9 && W > 3000);
+  if (!constant_ok) return u2 ? C2D_LS(2, FSRC_SMEM, 1, 0) : C2D_LS(1, FSRC_SMEM, 1, 0);
+  if (u2) return C2D_LS(2, FSRC_CONST, 1, 0);
+  if (W >= 4096) return C2D_LS(1, FSRC_CONST, 1, 1);
+  return C2D_LS(1, FSRC_CONST, 1, 2);
+#undef C2D_LS
+}
+
+// ------------------------------------------------------------------------------------------------
+// multi channel
+// ------------------------------------------------------------------------------------------------
+template <int K>
+struct MultiCfg {
+  static constexpr int FB = (K <= 4) ? 8 : (K <= 8 ? 4 : 2);
+};
+
+template <int K, int FB>
+int launch_multi_fb(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
+                    cudaStream_t stream, int band_h, const DevInfo &dev, size_t smem) {
+  auto kernel = k_conv2d_multi<K, FB>;
+  static std::atomic<int> occ_cache{0};
+  static std::atomic<int> smem_set{0};
+  if (smem > 48 * 1024 && smem_set.load() < static_cast<int>(smem)) {
+    if (cudaFuncSetAttribute(kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, dev.smem_optin) != cudaSuccess)
+      return CONV2D_ECUDA;
+    smem_set.store(dev.smem_optin);
+  }
+  MultiArgs a;
+  a.in = in;
+  a.filt = filt;
+  a.out = out;
+  a.N = N;
+  a.C = C;
+  a.H = H;
+  a.W = W;
+  a.F = F;
+  a.Ho = H - K + 1;
+  a.Wo = W - K + 1;
+  a.n_cb = ceil_div(a.Wo, 128);
+  a.n_fb = ceil_div(F, FB);
+  a.aligned = (aligned16(in) && (W % 4 == 0)) ? 1 : 0;
+  if (band_h <= 0) {
+    // occupancy of this instantiation with this smem size (the cache holds the value for the
+    // first smem size seen; good enough for choosing a band height)
+    const long long resident_warps =
+        static_cast<long long>(cta_occupancy(kernel, smem, occ_cache)) * kCtaWarps * dev.num_sms;
+    const long long groups = static_cast<long long>(N) * a.n_fb * a.n_cb;
+    long long bands = resident_warps / groups;
+    if (bands < 1) bands = 1;
+    band_h = ceil_div(a.Ho, bands);
+    const int min_band = 4;
+    if (band_h < min_band) band_h = min_band;
+  }
+  if (band_h > a.Ho) band_h = a.Ho;
+  a.band_h = band_h;
+  int n_bands = ceil_div(a.Ho, band_h);
+  // all 4 warps of a CTA must share (n, F-block): pad the tiles per (n, F-block) to a multiple of 4
+  while ((static_cast<long long>(a.n_cb) * n_bands) % kCtaWarps) ++n_bands;
+  a.n_bands = n_bands;
+  a.n_tiles = static_cast<long long>(N) * a.n_fb * n_bands * a.n_cb;
+  const long long blocks = (a.n_tiles + kCtaWarps - 1) / kCtaWarps;
+  if (blocks > 0x7fffffffLL) return CONV2D_ESHAPE;
+  kernel<<<static_cast<unsigned>(blocks), kCtaWarps * kWarp, smem, stream>>>(a);
+  return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
+}
+
+template <int K, int FB, int U, int SEG, int GUARDS, int PF>
+int launch_multi2_v(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
+                    cudaStream_t stream, int band_h, const DevInfo &dev) {
+  constexpr int KP = KCfg<K>::KP;
+  constexpr int SEGS = kWarp / SEG;
+  auto kernel = k_conv2d_multi2<K, FB, U, SEG, GUARDS, PF>;
+  static std::atomic<int> occ_cache{0};
+  static std::atomic<int> smem_set{0};
+  const size_t smem = static_cast<size_t>(C) * K * FB * KP * sizeof(float);
+  if (smem > static_cast<size_t>(dev.smem_optin)) return CONV2D_ESHAPE;
+  if (smem > 48 * 1024 && smem_set.load() == 0) {
+    if (cudaFuncSetAttribute(kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, dev.smem_optin) != cudaSuccess)
+      return CONV2D_ECUDA;
+    smem_set.store(1);
+  }
+  Multi2Args a;
+  a.in = in;
+  a.filt = filt;
+  a.out = out;
+  a.N = N;
+  a.C = C;
+  a.H = H;
+  a.W = W;
+  a.F = F;
+  a.Ho = H - K + 1;
+  a.Wo = W - K + 1;
+  a.n_cb = ceil_div(a.Wo, 4 * SEG * U);
+  a.n_fb = ceil_div(F, FB);
+  a.n_groups = ceil_div(N, SEGS);
+  a.aligned = (aligned16(in) && (W % 4 == 0)) ? 1 : 0;
+  if (band_h <= 0) {
+    // one full wave of resident warps
+    const long long resident_warps =
+        static_cast<long long>(cta_occupancy(kernel, smem, occ_cache)) * kCtaWarps * dev.num_sms;
+    const long long groups = static_cast<long long>(a.n_groups) * a.n_fb * a.n_cb;
+    long long bands = resident_warps / groups;
+    if (bands < 1) bands = 1;
+    band_h = ceil_div(a.Ho, bands);
+  }
+  if (band_h > a.Ho) band_h = a.Ho;
+  a.band_h = band_h;
+  int n_bands = ceil_div(a.Ho, band_h);
+  while ((static_cast<long long>(a.n_cb) * n_bands) % kCtaWarps) ++n_bands;
+  a.n_bands = n_bands;
+  a.n_tiles = static_cast<long long>(a.n_groups) * a.n_fb * n_bands * a.n_cb;
+  const long long blocks = (a.n_tiles + kCtaWarps - 1) / kCtaWarps;
+  if (blocks > 0x7fffffffLL) return CONV2D_ESHAPE;
+  kernel<<<static_cast<unsigned>(blocks), kCtaWarps * kWarp, smem, stream>>>(a);
+  return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
+}
+
+// fraction of a segment-row's lanes doing valid columns
+inline double lane_use(int Wo, int span) { return double(Wo) / (double(ceil_div(Wo, span)) * span); }
+
+template <int K>
+int launch_multi(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
+                 cudaStream_t stream, int band_h, const DevInfo &dev) {
+  // FB filters per warp (K*FB*4 accumulators); FBH = half of it (more warps, smaller loop body)
+  constexpr int FB = (K <= 3) ? 8 : (K <= 7 ? 4 : 2);
+  constexpr int FBH = (FB > 1) ? FB / 2 : 1;
+  constexpr int GUARDS = (K <= 5) ? 2 : 0;
+  constexpr int KP = KCfg<K>::KP;
+  const int Wo = W - K + 1;
+  const int mv = g_mvariant.load(std::memory_order_relaxed);
+  int rc = CONV2D_ESHAPE;
+  if (mv == 9) {  // the round-1 kernel
+    constexpr int LFB = MultiCfg<K>::FB;
+    const size_t lsmem = static_cast<size_t>(C) * K * LFB * KP * sizeof(float);
+    if (lsmem <= static_cast<size_t>(dev.smem_optin))
+      return launch_multi_fb<K, LFB>(in, N, C, H, W, filt, F, out, stream, band_h, dev, lsmem);
+  }
+#define C2D_LM(FBB, SEGG) \
+  launch_multi2_v<K, FBB, 1, SEGG, GUARDS, 2>(in, N, C, H, W, filt, F, out, stream, band_h, dev)
+  // Tuned on B200 (tools/multi_variants.py): 16-lane segments (two images per warp) unless they waste
+  // clearly more lanes than whole-warp rows -- more column blocks take the vector fast path and the
+  // ragged edge is a smaller share; FB = 8 filters per warp for K <= 3, half the register-limited FB
+  // above (smaller loop body, more resident warps).
+  const bool seg16 = (mv == 2 || mv == 4) || (mv == 0 && N >= 2 && lane_use(Wo, 64) >= lane_use(Wo, 128) - 0.05);
+  const bool half = (mv == 3 || mv == 4) || (mv == 0 && K > 3);
+  if (half)
+    rc = seg16 ? C2D_LM(FBH, 16) : C2D_LM(FBH, 32);
+  else
+    rc = seg16 ? C2D_LM(FB, 16) : C2D_LM(FB, 32);
+#undef C2D_LM
+  if (rc != CONV2D_ESHAPE) return rc;
+  // F-block does not fit shared memory: round-1 kernel with one filter per warp
+  const size_t smem1 = static_cast<size_t>(C) * K * KP * sizeof(float);
+  if (smem1 <= static_cast<size_t>(dev.smem_optin))
+    return launch_multi_fb<K, 1>(in, N, C, H, W, filt, F, out, stream, band_h, dev, smem1);
+  return CONV2D_ESHAPE;
+}
+
+}  // namespace
+
+namespace c2d {
+
+template <int K>
+int single_entry(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
+                 const DevInfo &dev) {
+  return launch_single<K>(in, H, W, filt, out, stream, band_h, dev);
+}
+
+template <int K>
+int multi_entry(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
+                cudaStream_t stream, int band_h, const DevInfo &dev) {
+  return launch_multi<K>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
+}
+
+}  // namespace c2d

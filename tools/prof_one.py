@@ -27,8 +27,10 @@ def main():
     ap.add_argument("--band", type=int, default=0)
     ap.add_argument("--time", action="store_true")
     ap.add_argument("--variant", type=int, default=0)
+    ap.add_argument("--mvariant", type=int, default=0)
     a = ap.parse_args()
     pkg._capi.debug_set_variant(a.variant)
+    pkg._capi.debug_set_multi_variant(a.mvariant)
     dev = torch.device("cuda")
     if a.kind == "single":
         S = [int(v) for v in a.shape.split(",")]
