@@ -12,13 +12,19 @@
  *
  * Conventions shared by every entry point
  *   - All tensor pointers are DEVICE pointers (global memory of the current CUDA device), owned by
- *     the caller. The library never allocates, frees, or retains them after the call returns.
+ *     the caller (except conv2d_single_host: host pointers). The library never frees or retains them
+ *     after the call returns.
  *   - fp32, dense, row-major: no strides, no padding; every pointer must be 4-byte aligned. Any
  *     width and any 4-byte alignment is supported; 16-byte-aligned inputs with W % 4 == 0 take the
  *     vectorised (LDG.128) path.
  *   - `stream` is a cudaStream_t passed as void* (NULL = legacy default stream). Work is enqueued
- *     asynchronously on it; there is no host synchronisation. The call is reentrant and thread-safe:
- *     filters are staged per CTA into shared memory, there is no module-global mutable state.
+ *     asynchronously on it; there is no host synchronisation. The calls are reentrant and
+ *     thread-safe. Single-channel filters are staged (a stream-ordered device-to-device copy) into a
+ *     per-K slot of the module's __constant__ bank; an event recorded behind each kernel orders the
+ *     next overwrite of the slot, so concurrent calls on different streams never see each other's
+ *     filter (same-K calls on different streams are serialised by that wait). Under CUDA-graph
+ *     capture the filter is staged per CTA in shared memory instead. Multi-channel filters are
+ *     staged per CTA in shared memory.
  *   - Return value: 0 when the work was enqueued. A negative CONV2D_E* code when an argument is
  *     invalid (nothing was launched) or the launch itself failed. Asynchronous execution errors
  *     surface at the caller's next synchronisation, as in CUDA.
@@ -44,6 +50,7 @@ extern "C" {
 #define CONV2D_EOVERLAP (-4)  /* the output range overlaps the input or the filter range */
 #define CONV2D_ECUDA (-5)     /* the kernel launch failed (cudaGetLastError after the launch) */
 #define CONV2D_EALIGN (-6)    /* a tensor pointer is not 4-byte aligned */
+#define CONV2D_EALLOC (-7)    /* device memory for a host-buffer call could not be allocated */
 
 #define CONV2D_MAX_K 15
 
@@ -62,8 +69,9 @@ int conv2d_single(const float *in, int H, int W, const float *filt, int K, float
  *   filt : F*C*K*K floats (FCKK == torch OIHW)
  *   out  : N*F*(H-K+1)*(W-K+1) floats (NFHoWo):
  *          out[n][f][y][x] = sum_{c<C} sum_{i<K} sum_{j<K} in[n][c][y+i][x+j] * filt[f][c][i][j]
- *   The filters of one F-block (all C channels) are staged in shared memory; F*C*K*K of any size
- *   is supported (the F-block is sized to fit).
+ *   The filters of one F-block (all C channels) are staged in shared memory; the F-block shrinks to
+ *   one filter when needed, so C*K*ceil(K/4)*4*4 bytes must fit in a CTA's shared memory (227 KiB:
+ *   e.g. C <= 236 at K = 15, C <= 4843 at K = 3); larger C returns CONV2D_ESHAPE.
  */
 int conv2d_multi(const float *in, int N, int C, int H, int W, const float *filt, int F, int K,
                  float *out, void *stream);
@@ -87,6 +95,22 @@ int conv2d_multi_ex(const float *in, int N, int C, int H, int W, const float *fi
  */
 int conv2d_single_direct(const float *in, int H, int W, const float *filt, int K, float *out,
                          void *stream);
+
+/*
+ * End-to-end single-channel call on HOST buffers (the user-facing path for data that lives in host
+ * memory): same operation and result as conv2d_single, but in, filt and out are host pointers (pinned
+ * memory -- cudaHostAlloc / cudaHostRegister -- lets the copies run asynchronously at full PCIe
+ * speed; pageable memory works but the copies become synchronous).
+ * The image is processed in row chunks through a three-stage pipeline on the current device: the
+ * host->device copy of chunk i+1, the kernel of chunk i and the device->host copy of chunk i-1 run
+ * concurrently (two internal copy streams plus `stream` for the kernels). Device memory for the image
+ * is taken from the stream-ordered allocator (cudaMallocAsync) and released when the work completes;
+ * the library retains nothing. All work is ordered after the work already enqueued on `stream`, and
+ * `stream` is ordered after all of it: synchronise `stream` before reading `out`.
+ * chunk_rows <= 0 chooses ~8 MiB input chunks.
+ */
+int conv2d_single_host(const float *in, int H, int W, const float *filt, int K, float *out, void *stream,
+                       int chunk_rows);
 
 /* Human-readable text for a return code (static storage, never NULL). */
 const char *conv2d_strerror(int code);

@@ -10,7 +10,7 @@ LIB_PATH = os.path.join(_PKG, "libconv2d.so")
 
 # every symbol include/conv2d.h declares
 EXPORTS = ("conv2d_single", "conv2d_multi", "conv2d_single_ex", "conv2d_multi_ex", "conv2d_single_direct",
-           "conv2d_strerror", "conv2d_version")
+           "conv2d_single_host", "conv2d_strerror", "conv2d_version")
 
 CONV2D_OK = 0
 CONV2D_ENULL = -1
@@ -19,6 +19,7 @@ CONV2D_EK = -3
 CONV2D_EOVERLAP = -4
 CONV2D_ECUDA = -5
 CONV2D_EALIGN = -6
+CONV2D_EALLOC = -7
 CONV2D_MAX_K = 15
 
 _lib = None
@@ -46,8 +47,9 @@ def load(path: str | None = None):
     L.conv2d_single_direct.argtypes = [P, I, I, P, I, P, P]
     L.conv2d_multi.argtypes = [P, I, I, I, I, P, I, I, P, P]
     L.conv2d_multi_ex.argtypes = [P, I, I, I, I, P, I, I, P, P, I]
+    L.conv2d_single_host.argtypes = [P, I, I, P, I, P, P, I]
     for f in ("conv2d_single", "conv2d_single_ex", "conv2d_single_direct", "conv2d_multi",
-              "conv2d_multi_ex", "conv2d_version"):
+              "conv2d_multi_ex", "conv2d_single_host", "conv2d_version"):
         getattr(L, f).restype = I
     L.conv2d_strerror.argtypes = [I]
     L.conv2d_strerror.restype = ctypes.c_char_p
@@ -83,6 +85,10 @@ def conv2d_multi(in_ptr, N, C, H, W, filt_ptr, F, K, out_ptr, stream=0) -> int:
 
 def conv2d_multi_ex(in_ptr, N, C, H, W, filt_ptr, F, K, out_ptr, stream=0, band_h=0) -> int:
     return load().conv2d_multi_ex(in_ptr, N, C, H, W, filt_ptr, F, K, out_ptr, stream, band_h)
+
+
+def conv2d_single_host(in_ptr, H, W, filt_ptr, K, out_ptr, stream=0, chunk_rows=0) -> int:
+    return load().conv2d_single_host(in_ptr, H, W, filt_ptr, K, out_ptr, stream, chunk_rows)
 
 
 def conv2d_version() -> int:

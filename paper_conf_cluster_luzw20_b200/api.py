@@ -89,17 +89,25 @@ def conv2d_multi(x: torch.Tensor, w: torch.Tensor, out: torch.Tensor | None = No
 
 
 def conv2d_single_host(x_host: torch.Tensor, f_host: torch.Tensor, device="cuda", stream=None,
-                       out_host: torch.Tensor | None = None) -> torch.Tensor:
-    """End-to-end call on host tensors (pinned for async copies): H2D, kernel, D2H on one stream."""
+                       out_host: torch.Tensor | None = None, chunk_rows: int = 0) -> torch.Tensor:
+    """End-to-end call on host tensors through the C ABI's pipelined host-buffer entry
+    (conv2d_single_host): chunked H2D / kernel / D2H overlap. Pin the tensors for full PCIe speed.
+    Returns out_host; the result is ready once `stream` (default: the current stream) is synchronised."""
+    if x_host.is_cuda or f_host.is_cuda:
+        raise TypeError("conv2d_single_host takes host tensors")
+    if x_host.dtype != torch.float32 or f_host.dtype != torch.float32:
+        raise TypeError("float32 tensors required")
+    x_host = x_host.contiguous()
+    f_host = f_host.contiguous()
+    H, W = x_host.shape
+    K = f_host.shape[0]
+    if out_host is None:
+        out_host = torch.empty((max(H - K + 1, 0), max(W - K + 1, 0)), dtype=torch.float32, pin_memory=True)
     dev = torch.device(device)
     s = stream if stream is not None else torch.cuda.current_stream(dev)
-    with torch.cuda.stream(s):
-        x = x_host.to(dev, non_blocking=True)
-        f = f_host.to(dev, non_blocking=True)
-        y = conv2d_single(x, f, stream=s)
-        if out_host is None:
-            out_host = torch.empty(y.shape, dtype=torch.float32, pin_memory=True)
-        out_host.copy_(y, non_blocking=True)
+    with torch.cuda.device(dev):
+        _capi.check(_capi.conv2d_single_host(x_host.data_ptr(), H, W, f_host.data_ptr(), K, out_host.data_ptr(),
+                                             int(s.cuda_stream), chunk_rows))
     return out_host
 
 

@@ -164,6 +164,7 @@ const char *conv2d_strerror(int code) {
     case CONV2D_EOVERLAP: return "output overlaps input or filter";
     case CONV2D_ECUDA: return "CUDA launch error";
     case CONV2D_EALIGN: return "a tensor pointer is not 4-byte aligned";
+    case CONV2D_EALLOC: return "device memory for a host-buffer call could not be allocated";
     default: return "unknown error code";
   }
 }

@@ -232,3 +232,22 @@ def test_concurrent_streams_different_filters(cuda_device):
     torch.cuda.synchronize()
     for f, y in zip(fs, outs):
         assert torch.equal(y, pkg.conv2d_single(x, f))
+
+
+@pytest.mark.parametrize("pinned", [True, False])
+def test_host_buffer_pipeline(cuda_device, pinned):
+    """conv2d_single_host (H2D / kernel / D2H chunk pipeline) equals the device-resident call bit for
+    bit, for chunk sizes that do and do not divide the output height."""
+    for (H, W, K) in [(1000, 777, 3), (517, 1024, 15), (40, 300, 7)]:
+        xh = synth.fill_np(H, synth.TAG_INPUT, (H, W), "img")
+        fh = synth.make_filter(K, K, "rand")[0, 0]
+        x = torch.from_numpy(xh)
+        f = torch.from_numpy(fh)
+        if pinned:
+            x = x.pin_memory()
+            f = f.pin_memory()
+        ref = pkg.conv2d_single(x.cuda(), f.cuda()).cpu()
+        for chunk in (0, 1, 7, 64, 10 ** 6):
+            out = pkg.conv2d_single_host(x, f, chunk_rows=chunk)
+            torch.cuda.synchronize()
+            assert torch.equal(out, ref), (H, W, K, chunk)
