@@ -58,6 +58,10 @@ __device__ __forceinline__ void stg4(float *p, float a, float b, float c, float 
   __stcs(reinterpret_cast<float4 *>(p), make_float4(a, b, c, d));
 }
 
+__device__ __forceinline__ void lds4_at(unsigned saddr, float &a, float &b, float &c, float &d) {
+  asm volatile("ld.shared.v4.f32 {%0, %1, %2, %3}, [%4];" : "=f"(a), "=f"(b), "=f"(c), "=f"(d) : "r"(saddr));
+}
+
 // LDS.128 that the compiler may not hoist out of the row loop (keeps the staged filters out of the
 // register file).
 __device__ __forceinline__ void lds4_volatile(const float *p, float &a, float &b, float &c, float &d) {
@@ -113,6 +117,56 @@ __device__ __forceinline__ void load_row_g(RowBuf<K, U> &b, const float *__restr
     }
   }
 }
+
+// cp.async (LDGSTS) row ring: each lane copies its own quads global -> shared and later reads back
+// only what it wrote itself, so deep prefetch costs no registers, no register copies and no
+// cross-lane synchronisation (cp.async.wait_group per thread is enough).
+__device__ __forceinline__ void cp_async16(unsigned saddr, const void *g) {
+  asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(saddr), "l"(g) : "memory");
+}
+__device__ __forceinline__ void cp_async_commit() { asm volatile("cp.async.commit_group;" ::: "memory"); }
+template <int N>
+__device__ __forceinline__ void cp_async_wait() {
+  asm volatile("cp.async.wait_group %0;" ::"n"(N) : "memory");
+}
+
+// NST stages x (U+1) quads (U chunk quads + the halo quad) x 32 lanes x 16 B per warp
+template <int K, int U, int SEG, int NST>
+struct RowRing {
+  static constexpr unsigned kStageBytes = (U + 1) * kWarp * 16;
+  static constexpr unsigned kBytes = NST * kStageBytes;
+  unsigned base;  // shared-window address of this warp's ring
+  int lane, sl;
+
+  // issue the copies of one row segment into `stage` (aligned rows; `clamp` on ragged edges)
+  __device__ __forceinline__ void issue(int stage, const float *__restrict__ rowp, int x0, int W, bool clamp) const {
+    constexpr int NE = KCfg<K>::NE;
+    const unsigned sb = base + stage * kStageBytes + lane * 16;
+#pragma unroll
+    for (int u = 0; u < U; ++u) {
+      int x = x0 + 4 * SEG * u + 4 * sl;
+      if (clamp) x = min(x, W - 4);
+      cp_async16(sb + u * kWarp * 16, rowp + x);
+    }
+    if constexpr (NE > 0) {
+      int xe = x0 + 4 * SEG * U + 4 * (sl % NE);
+      if (clamp) xe = min(xe, W - 4);
+      cp_async16(sb + U * kWarp * 16, rowp + xe);
+    }
+    cp_async_commit();
+  }
+  __device__ __forceinline__ void read(int stage, RowBuf<K, U> &b) const {
+    const unsigned sb = base + stage * kStageBytes + lane * 16;
+#pragma unroll
+    for (int u = 0; u < U; ++u) lds4_at(sb + u * kWarp * 16, b.a[u][0], b.a[u][1], b.a[u][2], b.a[u][3]);
+    if constexpr (KCfg<K>::NE > 0) {
+      lds4_at(sb + U * kWarp * 16, b.e[0], b.e[1], b.e[2], b.e[3]);
+    } else {
+#pragma unroll
+      for (int t = 0; t < 4; ++t) b.e[t] = 0.f;
+    }
+  }
+};
 
 template <int K, int U, bool SAFE>
 __device__ __forceinline__ void load_row(RowBuf<K, U> &b, const float *__restrict__ rowp, int x0, int W, int lane,
@@ -176,10 +230,6 @@ constexpr int kConstSlotFloats = 256;  // >= 15 rows x 16 (padded) floats
 // One slot per translation unit: every K is compiled in its own unit (csrc/inst_kNN.cu) and so in its
 // own module with its own constant bank; slot "K" of the design is this array in unit K.
 __constant__ __align__(16) float c_filt[kConstSlotFloats];
-
-__device__ __forceinline__ void lds4_at(unsigned saddr, float &a, float &b, float &c, float &d) {
-  asm volatile("ld.shared.v4.f32 {%0, %1, %2, %3}, [%4];" : "=f"(a), "=f"(b), "=f"(c), "=f"(d) : "r"(saddr));
-}
 
 template <int K, int FSRC>
 struct FilterSrc {

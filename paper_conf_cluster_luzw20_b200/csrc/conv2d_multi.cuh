@@ -79,9 +79,12 @@ __device__ __forceinline__ void row_step_multi(float (&acc)[K][FB][U][4], const 
   }
 }
 
-template <int K, int FB, int U, int SEG, int GUARDS, int PF, bool SAFE>
+// EDGE 0: interior tile (ring, vector stores); 1: aligned rows, ragged right edge (ring with clamped
+// addresses, masked scalar stores); 2: misaligned rows (guarded scalar loads in registers, masked stores)
+template <int K, int FB, int U, int SEG, int GUARDS, int PF, int EDGE>
 __device__ __forceinline__ void multi_tile2(const Multi2Args &a, const MultiFilter<K, FB> &mf, int n,
-                                            bool seg_active, int f0, int x0, int ob, int oe, int lane) {
+                                            bool seg_active, int f0, int x0, int ob, int oe, int lane,
+                                            unsigned ring_base) {
   const int sl = lane & (SEG - 1);
   const int C = a.C;
   const int rend = oe + K - 1;
@@ -98,31 +101,66 @@ __device__ __forceinline__ void multi_tile2(const Multi2Args &a, const MultiFilt
 #pragma unroll
         for (int v = 0; v < 4; ++v) acc[q][fb][u][v] = 0.f;
 
-  // the (row, channel) stream: (r, c) -> (r, c+1) -> ... -> (r+1, 0); PF = 1 or 2 entries in flight
-  auto row_ptr = [&](int r, int c) { return img + c * plane + static_cast<size_t>(r) * a.W; };
-  RowBuf<K, U> n1, n2;
-  int pr = ob, pc = 0;  // (row, channel) of the next load to issue
+  // the (row, channel) stream: (r, c) -> (r, c+1) -> ... -> (r+1, 0). PF >= 3 and aligned rows: a
+  // PF-stage cp.async ring in shared memory (PF-1 entries in flight); otherwise PF (1 or 2) entries
+  // in registers (misaligned rows: one).
+  constexpr bool SAFE = (EDGE != 0);
+  constexpr int NST = (PF >= 3 && EDGE != 2) ? PF : 1;
+  constexpr int RPF = (NST == 1 && PF == 2 && EDGE != 2) ? 2 : 1;  // register prefetch depth
+  static_assert(NST == 1 || (NST & (NST - 1)) == 0, "ring depth must be a power of two");
+  RowRing<K, U, SEG, (NST > 1 ? NST : 2)> ring;
+  ring.base = ring_base;
+  ring.lane = lane;
+  ring.sl = sl;
+  RowBuf<K, U> n1, n2;  // register path: PF (1 or 2) entries in flight
+  // next entry to fetch: pointer advanced by one channel plane per entry, by one row after C entries
+  const float *__restrict__ fetch_row0 = img + static_cast<size_t>(ob) * a.W;  // channel 0 of row pr
+  const float *__restrict__ fetch = fetch_row0;
+  int pr = ob, pc = 0;
+  int t = 0;  // entries consumed
   auto advance = [&]() {
     if (++pc == C) {
       pc = 0;
-      pr = min(pr + 1, rlast);
+      if (pr < rlast) {
+        ++pr;
+        fetch_row0 += a.W;
+      }
+      fetch = fetch_row0;
+    } else {
+      fetch += plane;
     }
   };
-  load_row_g<K, U, SEG, SAFE>(n1, row_ptr(pr, pc), x0, a.W, sl, a.aligned);
-  advance();
-  if constexpr (PF == 2) {
-    load_row_g<K, U, SEG, SAFE>(n2, row_ptr(pr, pc), x0, a.W, sl, a.aligned);
+  constexpr bool clamp = (EDGE == 1);
+  if constexpr (NST > 1) {
+#pragma unroll
+    for (int st = 0; st < NST - 1; ++st) {
+      ring.issue(st, fetch, x0, a.W, clamp);
+      advance();
+    }
+  } else {
+    load_row_g<K, U, SEG, SAFE>(n1, fetch, x0, a.W, sl, a.aligned);
     advance();
+    if constexpr (RPF == 2) {
+      load_row_g<K, U, SEG, SAFE>(n2, fetch, x0, a.W, sl, a.aligned);
+      advance();
+    }
   }
   auto stream_row = [&](int r, int qmin, int qmax, auto guard_tag) {
     constexpr bool G = decltype(guard_tag)::value;
     for (int c = 0; c < C; ++c) {
-      const RowBuf<K, U> cur = n1;
-      if constexpr (PF == 2) {
+      RowBuf<K, U> cur;
+      if constexpr (NST > 1) {
+        cp_async_wait<NST - 2>();
+        ring.read(t & (NST - 1), cur);
+        ring.issue((t + NST - 1) & (NST - 1), fetch, x0, a.W, clamp);  // the stage read at t-1
+        ++t;
+      } else if constexpr (RPF == 2) {
+        cur = n1;
         n1 = n2;
-        load_row_g<K, U, SEG, SAFE>(n2, row_ptr(pr, pc), x0, a.W, sl, a.aligned);
+        load_row_g<K, U, SEG, SAFE>(n2, fetch, x0, a.W, sl, a.aligned);
       } else {
-        load_row_g<K, U, SEG, SAFE>(n1, row_ptr(pr, pc), x0, a.W, sl, a.aligned);
+        cur = n1;
+        load_row_g<K, U, SEG, SAFE>(n1, fetch, x0, a.W, sl, a.aligned);
       }
       advance();
       float w[U][KCfg<K>::WN];
@@ -177,7 +215,7 @@ __device__ __forceinline__ void multi_tile2(const Multi2Args &a, const MultiFilt
 // Tiles are ordered ((group * n_fb + fblk) * n_bands + band) * n_cb + cb; the host pads n_bands so that
 // the CTA's warps share (group, fblk): the CTA stages that F-block's C*K*FB*KP floats once.
 template <int K, int FB, int U, int SEG, int GUARDS, int PF>
-__global__ void __launch_bounds__(kCtaWarps *kWarp) k_conv2d_multi2(const Multi2Args a) {
+__global__ void __launch_bounds__(kCtaWarps *kWarp, 3) k_conv2d_multi2(const Multi2Args a) {
   constexpr int KP = KCfg<K>::KP;
   extern __shared__ __align__(16) float smem[];
   const long long tile0 = static_cast<long long>(blockIdx.x) * kCtaWarps;
@@ -197,6 +235,9 @@ __global__ void __launch_bounds__(kCtaWarps *kWarp) k_conv2d_multi2(const Multi2
   MultiFilter<K, FB> mf;
   mf.sbase = static_cast<unsigned>(__cvta_generic_to_shared(smem));
   const int lane = threadIdx.x & (kWarp - 1);
+  // this warp's cp.async row ring, after the F-block (16-byte aligned: total is a multiple of 4)
+  const unsigned ring_base = mf.sbase + static_cast<unsigned>(total) * 4u +
+                             (threadIdx.x >> 5) * RowRing<K, U, SEG, (PF >= 3 ? PF : 2)>::kBytes;
   const long long tile = tile0 + (threadIdx.x >> 5);
   if (tile >= a.n_tiles) return;
   const int cb = static_cast<int>(tile % a.n_cb);
@@ -210,11 +251,13 @@ __global__ void __launch_bounds__(kCtaWarps *kWarp) k_conv2d_multi2(const Multi2
   const int n_raw = group * SEGS + lane / SEG;
   const bool seg_active = n_raw < a.N;
   const int n = seg_active ? n_raw : a.N - 1;  // idle segments recompute the last image, never store
-  const bool fast = a.aligned && (x0 + 4 * SEG * U + 4 * KCfg<K>::NE <= a.W);  // uniform per warp
-  if (fast)
-    multi_tile2<K, FB, U, SEG, GUARDS, PF, false>(a, mf, n, seg_active, f0, x0, ob, oe, lane);
+  const bool inside = x0 + 4 * SEG * U + 4 * KCfg<K>::NE <= a.W;  // uniform per warp
+  if (a.aligned && inside)
+    multi_tile2<K, FB, U, SEG, GUARDS, PF, 0>(a, mf, n, seg_active, f0, x0, ob, oe, lane, ring_base);
+  else if (a.aligned)
+    multi_tile2<K, FB, U, SEG, GUARDS, PF, 1>(a, mf, n, seg_active, f0, x0, ob, oe, lane, ring_base);
   else
-    multi_tile2<K, FB, U, SEG, GUARDS, PF, true>(a, mf, n, seg_active, f0, x0, ob, oe, lane);
+    multi_tile2<K, FB, U, SEG, GUARDS, PF, 2>(a, mf, n, seg_active, f0, x0, ob, oe, lane, ring_base);
 }
 
 }  // namespace c2d

@@ -220,7 +220,8 @@ int launch_multi2_v(const float *in, int N, int C, int H, int W, const float *fi
   auto kernel = k_conv2d_multi2<K, FB, U, SEG, GUARDS, PF>;
   static std::atomic<int> occ_cache{0};
   static std::atomic<int> smem_set{0};
-  const size_t smem = static_cast<size_t>(C) * K * FB * KP * sizeof(float);
+  const size_t ring = (PF >= 3) ? kCtaWarps * RowRing<K, U, SEG, PF>::kBytes : 0;
+  const size_t smem = static_cast<size_t>(C) * K * FB * KP * sizeof(float) + ring;
   if (smem > static_cast<size_t>(dev.smem_optin)) return CONV2D_ESHAPE;
   if (smem > 48 * 1024 && smem_set.load() == 0) {
     if (cudaFuncSetAttribute(kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, dev.smem_optin) != cudaSuccess)
@@ -283,8 +284,16 @@ int launch_multi(const float *in, int N, int C, int H, int W, const float *filt,
     if (lsmem <= static_cast<size_t>(dev.smem_optin))
       return launch_multi_fb<K, LFB>(in, N, C, H, W, filt, F, out, stream, band_h, dev, lsmem);
   }
+  // row prefetch: a 4-stage cp.async ring in shared memory for K >= 5; two entries in registers for
+  // K <= 3, where a (row, channel) entry carries few FMAs and the ring's per-entry cost dominates
+  constexpr int PF = (K <= 3) ? 2 : 4;
 #define C2D_LM(FBB, SEGG) \
-  launch_multi2_v<K, FBB, 1, SEGG, GUARDS, 2>(in, N, C, H, W, filt, F, out, stream, band_h, dev)
+  launch_multi2_v<K, FBB, 1, SEGG, GUARDS, PF>(in, N, C, H, W, filt, F, out, stream, band_h, dev)
+#define C2D_LM2(FBB, SEGG) \
+  launch_multi2_v<K, FBB, 2, SEGG, GUARDS, PF>(in, N, C, H, W, filt, F, out, stream, band_h, dev)
+  constexpr int FBQ = (FBH > 1) ? FBH / 2 : 1;
+  if (mv == 5) return C2D_LM2(FBH, 16);
+  if (mv == 6) return C2D_LM2(FBQ, 16);
   // Tuned on B200 (tools/multi_variants.py): 16-lane segments (two images per warp) unless they waste
   // clearly more lanes than whole-warp rows -- more column blocks take the vector fast path and the
   // ragged edge is a smaller share; FB = 8 filters per warp for K <= 3, half the register-limited FB
@@ -296,6 +305,7 @@ int launch_multi(const float *in, int N, int C, int H, int W, const float *filt,
   else
     rc = seg16 ? C2D_LM(FB, 16) : C2D_LM(FB, 32);
 #undef C2D_LM
+#undef C2D_LM2
   if (rc != CONV2D_ESHAPE) return rc;
   // F-block does not fit shared memory: round-1 kernel with one filter per warp
   const size_t smem1 = static_cast<size_t>(C) * K * KP * sizeof(float);
