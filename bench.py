@@ -388,6 +388,33 @@ def run_e2e(points, unit, args, device):
 
     import paper_conf_cluster_luzw20_b200 as pkg
 
+    # Keep the host side on the GPU's NUMA node: the pinned staging buffers are first-touched by
+    # this thread, so they land in memory local to the GPU's PCIe root (cross-socket DMA halves the
+    # copy bandwidth and made the number swing run to run). Restored afterwards.
+    old_aff = os.sched_getaffinity(0)
+    try:
+        import pynvml
+
+        pynvml.nvmlInit()
+        h = pynvml.nvmlDeviceGetHandleByIndex(device.index or 0)
+        words = pynvml.nvmlDeviceGetCpuAffinity(h, (os.cpu_count() + 63) // 64)
+        local = {w * 64 + b for w, m in enumerate(words) for b in range(64) if m >> b & 1}
+        local &= old_aff
+        if local:
+            os.sched_setaffinity(0, local)
+    except Exception:
+        pass
+    try:
+        return _run_e2e(points, unit, args, device)
+    finally:
+        os.sched_setaffinity(0, old_aff)
+
+
+def _run_e2e(points, unit, args, device):
+    import torch
+
+    import paper_conf_cluster_luzw20_b200 as pkg
+
     main = torch.cuda.current_stream(device)
     streams = [torch.cuda.Stream(device=device) for _ in range(2)]
     hx = [p.x.cpu().pin_memory() for p in points]
@@ -543,7 +570,7 @@ def main():
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
     ap.add_argument("--workload", default="sweep", choices=sorted(WORKLOAD_DESC))
-    ap.add_argument("--e2e-steps", type=int, default=2)
+    ap.add_argument("--e2e-steps", type=int, default=3)
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--cpu-budget", type=float, default=10.0)

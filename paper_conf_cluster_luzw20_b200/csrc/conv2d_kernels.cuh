@@ -370,10 +370,17 @@ __device__ __forceinline__ float *out_row(const SingleArgs &a, int o) {
 //        into basic blocks the scheduler cannot overlap).
 // Row r+1 (r+2 when PF == 2) is in flight from memory while row r is computed; the next-row index
 // is clamped, so the loop body has no branch besides the store.
-template <int K, int U, int FSRC, int PF, int GUARDS, bool SAFE>
+// EDGE 0: interior tile (vector loads / stores); 1: aligned rows, ragged right edge (clamped vector
+// loads, masked scalar stores); 2: misaligned rows (guarded scalar loads, masked stores).
+// PF 1/2: rows r+1 (r+2) in flight in registers; PF >= 3 (power of two, EDGE < 2): a PF-stage cp.async
+// ring in shared memory with PF-1 rows in flight (latency-bound short bands and HBM-bound small K).
+template <int K, int U, int FSRC, int PF, int GUARDS, int EDGE>
 __device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc<K, FSRC> &fs, int x0, int ob,
-                                            int oe, int lane) {
-  static_assert(PF == 1 || PF == 2, "prefetch depth 1 or 2 rows");
+                                            int oe, int lane, unsigned ring_base) {
+  constexpr bool SAFE = (EDGE != 0);
+  constexpr int NST = (PF >= 3 && EDGE != 2) ? PF : 1;
+  constexpr int RPF = (PF == 2 || (PF >= 3 && EDGE == 2)) ? ((PF == 2) ? 2 : 1) : 1;
+  static_assert(NST == 1 || (NST & (NST - 1)) == 0, "ring depth must be a power of two");
   const int rend = oe + K - 1;  // input rows [ob, rend)
   const int rlast = rend - 1;
   float acc[K][U][4];
@@ -383,16 +390,33 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc
     for (int u = 0; u < U; ++u)
 #pragma unroll
       for (int v = 0; v < 4; ++v) acc[q][u][v] = 0.f;
-  RowBuf<K, U> n1, n2;  // rows r+1 (and r+2 when PF == 2) in flight
-  load_row<K, U, SAFE>(n1, in_row(a, ob), x0, a.W, lane, a.aligned);
-  if (PF == 2) load_row<K, U, SAFE>(n2, in_row(a, min(ob + 1, rlast)), x0, a.W, lane, a.aligned);
-  // advance the in-flight rows: returns row r, issues the load of row r+PF (index clamped)
+  RowRing<K, U, kWarp, (NST > 1 ? NST : 2)> ring;
+  ring.base = ring_base;
+  ring.lane = lane;
+  ring.sl = lane;
+  constexpr bool clamp = (EDGE == 1);
+  RowBuf<K, U> n1, n2;  // register path: rows r+1 (and r+2 when RPF == 2) in flight
+  if constexpr (NST > 1) {
+#pragma unroll
+    for (int st = 0; st < NST - 1; ++st) ring.issue(st, in_row(a, min(ob + st, rlast)), x0, a.W, clamp);
+  } else {
+    load_row<K, U, SAFE>(n1, in_row(a, ob), x0, a.W, lane, a.aligned);
+    if (RPF == 2) load_row<K, U, SAFE>(n2, in_row(a, min(ob + 1, rlast)), x0, a.W, lane, a.aligned);
+  }
+  // returns row r and issues the fetch of row r+depth (index clamped)
   auto next_row = [&](int r) {
-    const RowBuf<K, U> cur = n1;
-    if constexpr (PF == 2) {
+    RowBuf<K, U> cur;
+    if constexpr (NST > 1) {
+      cp_async_wait<NST - 2>();
+      const int k = r - ob;
+      ring.read(k & (NST - 1), cur);
+      ring.issue((k + NST - 1) & (NST - 1), in_row(a, min(r + NST - 1, rlast)), x0, a.W, clamp);
+    } else if constexpr (RPF == 2) {
+      cur = n1;
       n1 = n2;
       load_row<K, U, SAFE>(n2, in_row(a, min(r + 2, rlast)), x0, a.W, lane, a.aligned);
     } else {
+      cur = n1;
       load_row<K, U, SAFE>(n1, in_row(a, min(r + 1, rlast)), x0, a.W, lane, a.aligned);
     }
     return cur;
@@ -438,6 +462,7 @@ template <int K, int U, int FSRC, int CTAW, int PF = 1, int GUARDS = 0>
 __global__ void __launch_bounds__(CTAW *kWarp) k_conv2d_single(const SingleArgs a) {
   constexpr int KP = KCfg<K>::KP;
   __shared__ __align__(16) float sf[(FSRC == FSRC_SMEM) ? K * KP : 4];
+  extern __shared__ __align__(16) float ring_smem[];  // PF >= 3: CTAW rings of RowRing::kBytes
   FilterSrc<K, FSRC> fs;
   if constexpr (FSRC == FSRC_CONST) {
     fs.cbase = c_filt;
@@ -450,20 +475,24 @@ __global__ void __launch_bounds__(CTAW *kWarp) k_conv2d_single(const SingleArgs 
     fs.sbase = static_cast<unsigned>(__cvta_generic_to_shared(sf));
   }
   const int lane = threadIdx.x & (kWarp - 1);
-  const int tile = (CTAW == 1) ? static_cast<int>(blockIdx.x)
-                               : static_cast<int>(blockIdx.x) * CTAW + static_cast<int>(threadIdx.x >> 5);
+  const int warp = (CTAW == 1) ? 0 : static_cast<int>(threadIdx.x >> 5);
+  const int tile = static_cast<int>(blockIdx.x) * CTAW + warp;
   if (tile >= a.n_tiles) return;
+  const unsigned ring_base = static_cast<unsigned>(__cvta_generic_to_shared(ring_smem)) +
+                             warp * RowRing<K, U, kWarp, (PF >= 3 ? PF : 2)>::kBytes;
   const int cb = tile % a.n_cb;
   const int band = tile / a.n_cb;
   const int x0 = cb * 128 * U;
   const int ob = band * a.band_h;
   const int oe = min(ob + a.band_h, a.Ho);
   // fast tiles: 16B-aligned rows, every column of the tile and its extra halo quad in range
-  const bool fast = a.aligned && (x0 + 128 * U + 4 * KCfg<K>::NE <= a.W);  // warp-uniform
-  if (fast)
-    single_tile<K, U, FSRC, PF, GUARDS, false>(a, fs, x0, ob, oe, lane);
+  const bool inside = x0 + 128 * U + 4 * KCfg<K>::NE <= a.W;  // warp-uniform
+  if (a.aligned && inside)
+    single_tile<K, U, FSRC, PF, GUARDS, 0>(a, fs, x0, ob, oe, lane, ring_base);
+  else if (a.aligned)
+    single_tile<K, U, FSRC, PF, GUARDS, 1>(a, fs, x0, ob, oe, lane, ring_base);
   else
-    single_tile<K, U, FSRC, PF, GUARDS, true>(a, fs, x0, ob, oe, lane);
+    single_tile<K, U, FSRC, PF, GUARDS, 2>(a, fs, x0, ob, oe, lane, ring_base);
 }
 
 // ------------------------------------------------------------------------------------------------

@@ -93,6 +93,7 @@ int launch_single_v(const float *in, int H, int W, const float *filt, float *out
   constexpr int CTAW = (FSRC == FSRC_CONST) ? 1 : kCtaWarps;
   auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS>;
   static std::atomic<int> occ_cache{0};
+  const size_t ring = (PF >= 3) ? CTAW * RowRing<K, U, kWarp, (PF >= 3 ? PF : 2)>::kBytes : 0;
   SingleArgs a;
   a.in = in;
   a.filt = filt;
@@ -106,7 +107,7 @@ int launch_single_v(const float *in, int H, int W, const float *filt, float *out
   if (band_h <= 0) {
     // one full wave of warp tiles: bands = resident warps / column blocks
     const long long resident_warps =
-        static_cast<long long>(cta_occupancy(kernel, 0, occ_cache, CTAW)) * CTAW * dev.num_sms;
+        static_cast<long long>(cta_occupancy(kernel, ring, occ_cache, CTAW)) * CTAW * dev.num_sms;
     const long long bands = resident_warps / a.n_cb > 0 ? resident_warps / a.n_cb : 1;
     band_h = ceil_div(a.Ho, bands);
     if (band_h < min_band) band_h = min_band;
@@ -117,7 +118,7 @@ int launch_single_v(const float *in, int H, int W, const float *filt, float *out
   a.n_tiles = a.n_cb * n_bands;
   const int blocks = ceil_div(a.n_tiles, CTAW);
   auto go = [&]() {
-    kernel<<<blocks, CTAW * kWarp, 0, stream>>>(a);
+    kernel<<<blocks, CTAW * kWarp, ring, stream>>>(a);
     return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
   };
   if constexpr (FSRC == FSRC_CONST) return with_const_filter(filt, K, KCfg<K>::KP, stream, go);
@@ -140,17 +141,32 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
     case 4: if (constant_ok) return C2D_LS(2, FSRC_CONST, 1, 0); break;
     case 5: if (constant_ok) return C2D_LS(1, FSRC_CONST, 1, 1); break;
     case 6: if (constant_ok) return C2D_LS(1, FSRC_CONST, 1, 2); break;
+    case 7: if (constant_ok) return C2D_LS(2, FSRC_CONST, 4, 0); break;
+    case 8: if (constant_ok) return C2D_LS(2, FSRC_CONST, 8, 0); break;
+    case 9: if (constant_ok) return C2D_LS(1, FSRC_CONST, 4, 2); break;
     default: break;
   }
-  // Tuned on B200 (tools/variants.py, profiles/): two 128-column
-  // chunks per warp while K <= 7 (K = 9 on wide images); above, one chunk with a guarded prologue on
-  // wide images (tall bands) and guarded prologue + epilogue on narrow ones (short bands, where the
-  // wasted FMAs of an unguarded epilogue would be a large fraction).
-  const bool u2 = (K <= 7) || (K <= 9 && W > 3000);
-  if (!constant_ok) return u2 ? C2D_LS(2, FSRC_SMEM, 1, 0) : C2D_LS(1, FSRC_SMEM, 1, 0);
-  if (u2) return C2D_LS(2, FSRC_CONST, 1, 0);
-  if (W >= 4096) return C2D_LS(1, FSRC_CONST, 1, 1);
-  return C2D_LS(1, FSRC_CONST, 1, 2);
+  // Tuned on B200 (tools/variants.py sweeps):
+  //   K <= 5        two 128-column chunks per warp; row fetch from a 4-stage cp.async ring, except
+  //                 K <= 3 on wide images (one register row in flight is enough when HBM-bound);
+  //   K = 6..9      wide images (W >= 8192): two chunks + ring; narrower: one chunk + ring with
+  //                 Alg. 2 case-1/3 guards (short bands);
+  //   K = 10, 11    one chunk + ring + guards;
+  //   K >= 12       one chunk, register row fetch, guarded prologue on wide images (tall bands),
+  //                 guarded prologue + epilogue on narrow ones.
+  if (!constant_ok) return (K <= 7) ? C2D_LS(2, FSRC_SMEM, 1, 0) : C2D_LS(1, FSRC_SMEM, 1, 0);
+  if constexpr (K <= 5) {
+    if (K <= 3 && W > 1024) return C2D_LS(2, FSRC_CONST, 1, 0);
+    return C2D_LS(2, FSRC_CONST, 4, 0);
+  } else if constexpr (K <= 9) {
+    if (W >= 8192) return C2D_LS(2, FSRC_CONST, 4, 0);
+    return C2D_LS(1, FSRC_CONST, 4, 2);
+  } else if constexpr (K <= 11) {
+    return C2D_LS(1, FSRC_CONST, 4, 2);
+  } else {
+    if (W >= 4096) return C2D_LS(1, FSRC_CONST, 1, 1);
+    return C2D_LS(1, FSRC_CONST, 1, 2);
+  }
 #undef C2D_LS
 }
 
