@@ -112,6 +112,17 @@ int conv2d_single_direct(const float *in, int H, int W, const float *filt, int K
 int conv2d_single_host(const float *in, int H, int W, const float *filt, int K, float *out, void *stream,
                        int chunk_rows);
 
+/*
+ * Tensor-core variant of conv2d_multi for the large-C dense contraction (a separate, measured
+ * variant: BASELINE.json north_star). Same arguments, layouts and result contract as
+ * conv2d_multi; computed as an implicit GEMM (pixels x filters x C*K*K) on tcgen05 tensor cores with
+ * the 3xTF32 split (a = a_hi + a_lo; A_hi B_hi + A_hi B_lo + A_lo B_hi, fp32 accumulation in TMEM),
+ * within the same 1e-5 * sum|x||w| acceptance but NOT bitwise equal to conv2d_multi (different
+ * summation order and per-product rounding).
+ */
+int conv2d_multi_tc(const float *in, int N, int C, int H, int W, const float *filt, int F, int K, float *out,
+                    void *stream);
+
 /* Human-readable text for a return code (static storage, never NULL). */
 const char *conv2d_strerror(int code);
 

@@ -7,8 +7,8 @@ The product is libconv2d.so (C ABI, include/conv2d.h). This package is its thin 
     shard   multi-GPU partitioning: batch, filter and row-band (with a (K-1)-row NCCL halo)
 """
 from . import _capi
-from .api import (conv2d_multi, conv2d_multi_host, conv2d_single, conv2d_single_direct,
+from .api import (conv2d_multi, conv2d_multi_host, conv2d_multi_tc, conv2d_single, conv2d_single_direct,
                   conv2d_single_host)
 
-__all__ = ["_capi", "conv2d_multi", "conv2d_multi_host", "conv2d_single", "conv2d_single_direct",
-           "conv2d_single_host"]
+__all__ = ["_capi", "conv2d_multi", "conv2d_multi_host", "conv2d_multi_tc", "conv2d_single",
+           "conv2d_single_direct", "conv2d_single_host"]

@@ -88,6 +88,22 @@ def conv2d_multi(x: torch.Tensor, w: torch.Tensor, out: torch.Tensor | None = No
     return out
 
 
+def conv2d_multi_tc(x: torch.Tensor, w: torch.Tensor, out: torch.Tensor | None = None, stream=None) -> torch.Tensor:
+    """Tensor-core (tcgen05, 3xTF32) variant of conv2d_multi for the large-C dense contraction."""
+    _check_dev(x, "x")
+    _check_dev(w, "w")
+    if x.dim() != 4 or w.dim() != 4 or w.shape[1] != x.shape[1] or w.shape[2] != w.shape[3]:
+        raise ValueError("x must be (N, C, H, W) and w (F, C, K, K)")
+    N, C, H, W = x.shape
+    F, _, K, _ = w.shape
+    if out is None:
+        out = torch.empty((N, F, max(H - K + 1, 0), max(W - K + 1, 0)), dtype=torch.float32, device=x.device)
+    with torch.cuda.device(x.device):
+        _capi.check(_capi.conv2d_multi_tc(x.data_ptr(), N, C, H, W, w.data_ptr(), F, K, out.data_ptr(),
+                                          _stream_handle(stream)))
+    return out
+
+
 def conv2d_single_host(x_host: torch.Tensor, f_host: torch.Tensor, device="cuda", stream=None,
                        out_host: torch.Tensor | None = None, chunk_rows: int = 0) -> torch.Tensor:
     """End-to-end call on host tensors through the C ABI's pipelined host-buffer entry

@@ -93,3 +93,25 @@ def test_table1_layers(cuda_device, layer):
         x = dev_image((4, C, S, S), "img", seed=S + C)
         w = _w(F, C, K, "he", seed=F)
         check_full_multi(x, w, pkg.conv2d_multi(x, w))
+
+
+@pytest.mark.parametrize("shape", [(2, 64, 56, 56, 64, 3), (1, 3, 40, 45, 16, 5), (2, 16, 20, 37, 100, 3),
+                                   (1, 8, 33, 30, 64, 7), (3, 1, 28, 28, 32, 3), (1, 4, 19, 21, 256, 1)])
+def test_tensor_core_variant(cuda_device, shape):
+    """conv2d_multi_tc (tcgen05 3xTF32 implicit GEMM) meets the same 1e-5*sum|x||w| acceptance."""
+    N, C, H, W, F, K = shape
+    x = dev_image((N, C, H, W), "sym", seed=C + F)
+    w = _w(F, C, K, "he", seed=F)
+    check_full_multi(x, w, pkg.conv2d_multi_tc(x, w))
+
+
+def test_tensor_core_variant_config2_sampled(cuda_device):
+    """configs[2] at full size through the tensor-core variant, sampled outputs."""
+    N, C, F, S, K = 32, 64, 64, 56, 3
+    x = dev_image((N, C, S, S), "sym", seed=synth.BASE_SEED + 2)
+    w = _w(F, C, K, "he", seed=synth.BASE_SEED + 2)
+    y = pkg.conv2d_multi_tc(x, w)
+    rng = np.random.default_rng(22)
+    P = 800
+    check_points_multi(x, w, y, rng.integers(0, N, P), rng.integers(0, F, P), rng.integers(0, S - K + 1, P),
+                       rng.integers(0, S - K + 1, P))
