@@ -46,9 +46,15 @@ def load_peaks():
         with open(p) as fh:
             d = json.load(fh)
         return {"hbm_gbs": float(d["hbm_gbs"]), "sm_max_mhz": float(d.get("sm_max_mhz", 1965.0)),
+                "bf16_tflops": float(d.get("bf16_tflops", 1590.0)),
                 "source": "measured (MEASURED_PEAKS.json)"}
     except Exception:
-        return {"hbm_gbs": 6650.0, "sm_max_mhz": 1965.0, "source": "fallback (B200_PROFILING.md)"}
+        return {"hbm_gbs": 6650.0, "sm_max_mhz": 1965.0, "bf16_tflops": 1590.0,
+                "source": "fallback (B200_PROFILING.md)"}
+
+
+# nominal dense tf32 / bf16 tensor throughput ratio (B200_PROFILING.md: 1.1 vs 2.25 PFLOP/s)
+TF32_PER_BF16 = 1.1 / 2.25
 
 
 def fp32_fma_peak_tflops(sm_mhz):
@@ -117,8 +123,16 @@ def workload_points(name):
         return [Point("multi", "N128 C3 F64 224^2 K7", (128, 3, 224, 224, 64), 7)], "GFLOP/s"
     if name == "config4":
         return [Point("single", "32768^2 K=15", (32768, 32768), 15)], "Gpixel/s"
+    if name == "table1":  # PAPER.md Table I: 11 layers x C in {1, 3}, N = 128
+        return [Point("multi", f"{nm} C{C} N128 {S}^2 F{F} K{K}", (128, C, S, S, F), K)
+                for C in (1, 3) for nm, S, F, K in TABLE1], "GFLOP/s"
     raise SystemExit(f"unknown workload {name}")
 
+
+# PAPER.md Table I: name, IH = IW, FN, FH = FW
+TABLE1 = [("CONV1", 28, 128, 3), ("CONV2", 56, 64, 3), ("CONV3", 12, 64, 5), ("CONV4", 14, 16, 5),
+          ("CONV5", 24, 256, 5), ("CONV6", 24, 64, 5), ("CONV7", 28, 16, 5), ("CONV8", 28, 512, 3),
+          ("CONV9", 56, 256, 3), ("CONV10", 112, 128, 3), ("CONV11", 224, 64, 3)]
 
 WORKLOAD_DESC = {
     "sweep": "BASELINE.json configs[1]: single-channel sweep, 1024^2/2048^2/4096^2/8192^2 x K in "
@@ -127,6 +141,7 @@ WORKLOAD_DESC = {
     "config2": "BASELINE.json configs[2]: N=32, C=F=64, 56x56, K=3",
     "config3": "BASELINE.json configs[3]: N=128, C=3, F=64, 224x224, K=7",
     "config4": "BASELINE.json configs[4]: 32768x32768, K=15 (row bands + NCCL halo at N>1)",
+    "table1": "PAPER.md Table I (P:335-352): 11 layers x C in {1,3}, N=128 (22 conv2d_multi calls per step)",
 }
 
 
@@ -252,6 +267,8 @@ def run_ours(args):
             shard.rowband_conv2d_single(p.x, p.f, band, p.y)
         elif p.kind == "single":
             pkg.conv2d_single(p.x, p.f, out=p.y, stream=stream)
+        elif args.multi_impl == "tc":
+            pkg.conv2d_multi_tc(p.x, p.f, out=p.y, stream=stream)
         else:
             pkg.conv2d_multi(p.x, p.f, out=p.y, stream=stream)
 
@@ -323,16 +340,23 @@ def run_ours(args):
     dp = points[dom]
     dkind, _ = dp.bound(peaks, sm_mhz_peak)
     dsec = dom_ms * 1e-3
-    if dkind == "hbm":
+    if dp.kind == "multi" and args.multi_impl == "tc":
+        # tensor-core variant: the executed TF32 MMA flops (3 per useful product, the 3xTF32 split)
+        # against the tf32 tensor peak (measured bf16 burst x the nominal tf32/bf16 ratio)
+        roof = {"bound": "tensor", "achieved": 3 * dp.flops / dsec / 1e12,
+                "peak": peaks["bf16_tflops"] * TF32_PER_BF16, "unit": "TFLOP/s",
+                "note": "executed tf32 MMA TFLOP/s = 3 x useful (3xTF32); peak = bf16 burst x 1.1/2.25"}
+    elif dkind == "hbm":
         roof = {"bound": "hbm", "achieved": dp.bytes / dsec / 1e9, "peak": peaks["hbm_gbs"], "unit": "GB/s"}
     else:
         roof = {"bound": "alu", "achieved": dp.flops / dsec / 1e12, "peak": fp32_fma_peak_tflops(sm_mhz_peak),
                 "unit": "TFLOP/s"}
     roof["frac"] = roof["achieved"] / roof["peak"]
-    roof["kernel"] = f"conv2d_{dp.kind} {dp.name}"
+    roof["kernel"] = (f"conv2d_multi_tc {dp.name}" if dp.kind == "multi" and args.multi_impl == "tc"
+                      else f"conv2d_{dp.kind} {dp.name}")
     roof["share_of_step"] = dom_ms / max(total_ms / args.steps, 1e-12)
     roof["launch_ms"] = round(dom_ms, 5)
-    roof["peak_source"] = (peaks["source"] if dkind == "hbm" else
+    roof["peak_source"] = (peaks["source"] if dkind == "hbm" or roof["bound"] == "tensor" else
                            f"fp32 FMA: 148 SM x 128 lanes x 2 x {sm_mhz_peak:.0f} MHz (sm_max_mhz, "
                            f"{peaks['source']})")
     roof["traffic"] = load_traffic(dp)
@@ -361,6 +385,7 @@ def run_ours(args):
         "dtype": "f32",
         "data": "synthetic (seeded counter-based generator, gen/synth.py)",
         "config": {"workload": WORKLOAD_DESC[args.workload],
+                   **({"multi_impl": args.multi_impl} if points[0].kind == "multi" else {}),
                    "l2": "512 MiB write between timed steps (outside the events) + distinct buffers per "
                          "conv; 8192^2 inputs also exceed L2",
                    "parallelism": ("row bands + NCCL halo" if rowband else
@@ -446,8 +471,10 @@ def _run_e2e(points, unit, args, device):
             s.wait_stream(main)
         for i, p in enumerate(points):
             s = streams[i % 2]
-            fn = pkg.conv2d_single_host if p.kind == "single" else pkg.conv2d_multi_host
-            fn(hx[i], hf[i], device=device, stream=s, out_host=hy[i])
+            if p.kind == "single":
+                pkg.conv2d_single_host(hx[i], hf[i], device=device, stream=s, out_host=hy[i])
+            else:
+                pkg.conv2d_multi_host(hx[i], hf[i], device=device, stream=s, out_host=hy[i], impl=args.multi_impl)
         for s in streams:
             main.wait_stream(s)
 
@@ -466,7 +493,8 @@ def _run_e2e(points, unit, args, device):
     d2h = sum(4 * p.y.numel() for p in points)
     return {"value": round(units / (ms * 1e-3) / 1e9, 3), "unit": unit, "h2d_bytes_per_step": h2d,
             "d2h_bytes_per_step": d2h, "steps": steps, "ms_per_step": round(ms / steps, 3),
-            "path": "conv2d_single_host (C ABI, pinned host buffers, 2 streams)"}
+            "path": ("conv2d_single_host (C ABI, pinned host buffers, 2 streams)" if points[0].kind == "single"
+                     else f"conv2d_multi_host (impl={args.multi_impl}; pinned host buffers, 2 streams)")}
 
 
 def load_traffic(p):
@@ -596,6 +624,8 @@ def main():
     ap.add_argument("--cpu-budget", type=float, default=10.0)
     ap.add_argument("--ref-budget", type=float, default=90.0)
     ap.add_argument("--variant", type=int, default=0, help="tuning: force a single-channel kernel variant")
+    ap.add_argument("--multi-impl", choices=["cuda", "tc"], default="cuda",
+                    help="multi-channel workloads: conv2d_multi (CUDA cores) or conv2d_multi_tc (tcgen05 3xTF32)")
     args = ap.parse_args()
     if args.warmup < 3 and args.impl == "ours":
         args.warmup = 3  # contract: W >= 3

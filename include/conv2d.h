@@ -104,8 +104,8 @@ int conv2d_single_direct(const float *in, int H, int W, const float *filt, int K
  * The image is processed in row chunks through a three-stage pipeline on the current device: the
  * host->device copy of chunk i+1, the kernel of chunk i and the device->host copy of chunk i-1 run
  * concurrently (two internal copy streams plus `stream` for the kernels). Device memory for the image
- * is taken from the stream-ordered allocator (cudaMallocAsync) and released when the work completes;
- * the library retains nothing. All work is ordered after the work already enqueued on `stream`, and
+ * is taken from the library's stream-ordered scratch pool (see conv2d_release_scratch) and returned
+ * to it when the work completes. All work is ordered after the work already enqueued on `stream`, and
  * `stream` is ordered after all of it: synchronise `stream` before reading `out`.
  * chunk_rows <= 0 chooses ~8 MiB input chunks.
  */
@@ -118,10 +118,21 @@ int conv2d_single_host(const float *in, int H, int W, const float *filt, int K, 
  * conv2d_multi; computed as an implicit GEMM (pixels x filters x C*K*K) on tcgen05 tensor cores with
  * the 3xTF32 split (a = a_hi + a_lo; A_hi B_hi + A_hi B_lo + A_lo B_hi, fp32 accumulation in TMEM),
  * within the same 1e-5 * sum|x||w| acceptance but NOT bitwise equal to conv2d_multi (different
- * summation order and per-product rounding).
+ * summation order and per-product rounding). The filters are split into hi/lo tensor-core tiles in a
+ * stream-ordered scratch buffer from the library's pool (2 * ceil(F/FN)*FN * ceil(C*K*K/32)*32 floats,
+ * FN in {32, 64, 128, 256}); CONV2D_EALLOC if that fails. Limits: C*H*W < 2^31 and C*K*K <= 16384
+ * (CONV2D_ESHAPE otherwise).
  */
 int conv2d_multi_tc(const float *in, int N, int C, int H, int W, const float *filt, int F, int K, float *out,
                     void *stream);
+
+/*
+ * The library's stream-ordered scratch pool (conv2d_single_host buffers, conv2d_multi_tc filter
+ * tiles) keeps freed memory for reuse by later calls, like a caching allocator. This call releases
+ * the unused part of the current device's pool back to the driver (memory still in use by enqueued
+ * work is kept). Returns 0, or CONV2D_ECUDA.
+ */
+int conv2d_release_scratch(void);
 
 /* Human-readable text for a return code (static storage, never NULL). */
 const char *conv2d_strerror(int code);

@@ -10,7 +10,7 @@ LIB_PATH = os.path.join(_PKG, "libconv2d.so")
 
 # every symbol include/conv2d.h declares
 EXPORTS = ("conv2d_single", "conv2d_multi", "conv2d_single_ex", "conv2d_multi_ex", "conv2d_single_direct",
-           "conv2d_single_host", "conv2d_multi_tc", "conv2d_strerror", "conv2d_version")
+           "conv2d_single_host", "conv2d_multi_tc", "conv2d_release_scratch", "conv2d_strerror", "conv2d_version")
 
 CONV2D_OK = 0
 CONV2D_ENULL = -1
@@ -49,8 +49,10 @@ def load(path: str | None = None):
     L.conv2d_multi_ex.argtypes = [P, I, I, I, I, P, I, I, P, P, I]
     L.conv2d_single_host.argtypes = [P, I, I, P, I, P, P, I]
     L.conv2d_multi_tc.argtypes = [P, I, I, I, I, P, I, I, P, P]
+    L.conv2d_release_scratch.argtypes = []
     for f in ("conv2d_single", "conv2d_single_ex", "conv2d_single_direct", "conv2d_multi",
-              "conv2d_multi_ex", "conv2d_single_host", "conv2d_multi_tc", "conv2d_version"):
+              "conv2d_multi_ex", "conv2d_single_host", "conv2d_multi_tc", "conv2d_release_scratch",
+              "conv2d_version"):
         getattr(L, f).restype = I
     L.conv2d_strerror.argtypes = [I]
     L.conv2d_strerror.restype = ctypes.c_char_p
@@ -94,6 +96,10 @@ def conv2d_single_host(in_ptr, H, W, filt_ptr, K, out_ptr, stream=0, chunk_rows=
 
 def conv2d_multi_tc(in_ptr, N, C, H, W, filt_ptr, F, K, out_ptr, stream=0) -> int:
     return load().conv2d_multi_tc(in_ptr, N, C, H, W, filt_ptr, F, K, out_ptr, stream)
+
+
+def conv2d_release_scratch() -> int:
+    return load().conv2d_release_scratch()
 
 
 def conv2d_version() -> int:

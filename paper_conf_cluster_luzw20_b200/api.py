@@ -128,13 +128,17 @@ def conv2d_single_host(x_host: torch.Tensor, f_host: torch.Tensor, device="cuda"
 
 
 def conv2d_multi_host(x_host: torch.Tensor, w_host: torch.Tensor, device="cuda", stream=None,
-                      out_host: torch.Tensor | None = None) -> torch.Tensor:
+                      out_host: torch.Tensor | None = None, impl: str = "cuda") -> torch.Tensor:
+    """Host tensors in and out around conv2d_multi (impl="cuda", CUDA cores) or conv2d_multi_tc
+    (impl="tc", tensor cores), all on one stream."""
+    if impl not in ("cuda", "tc"):
+        raise ValueError("impl must be 'cuda' or 'tc'")
     dev = torch.device(device)
     s = stream if stream is not None else torch.cuda.current_stream(dev)
     with torch.cuda.stream(s):
         x = x_host.to(dev, non_blocking=True)
         w = w_host.to(dev, non_blocking=True)
-        y = conv2d_multi(x, w, stream=s)
+        y = (conv2d_multi_tc if impl == "tc" else conv2d_multi)(x, w, stream=s)
         if out_host is None:
             out_host = torch.empty(y.shape, dtype=torch.float32, pin_memory=True)
         out_host.copy_(y, non_blocking=True)

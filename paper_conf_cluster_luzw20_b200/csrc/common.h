@@ -20,6 +20,13 @@ extern std::atomic<int> g_variant;    // single-channel kernel variant
 extern std::atomic<int> g_min_band;   // minimum band height of the automatic band choice
 extern std::atomic<int> g_mvariant;   // multi-channel kernel variant
 
+// Stream-ordered scratch memory from a library-owned memory pool of the current device (release
+// threshold "never", so the pool keeps its memory across synchronisations instead of returning it to
+// the driver -- the default pool trims at every sync, which turns each call into a real allocation).
+// Release with cudaFreeAsync on a stream ordered after the last use.
+cudaError_t scratch_alloc(void **p, size_t bytes, cudaStream_t stream);
+cudaError_t scratch_trim();
+
 // per-K entry points, explicitly instantiated one K per translation unit (csrc/inst_kNN.cu)
 template <int K>
 int single_entry(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,

@@ -29,6 +29,49 @@ __global__ void __launch_bounds__(256) k_conv2d_direct(const float *__restrict__
   out[idx] = s;
 }
 
+// ------------------------------------------------------------------------------------------------
+// library-owned stream-ordered scratch pool, one per device
+// ------------------------------------------------------------------------------------------------
+namespace {
+constexpr int kPoolDevices = 64;
+std::mutex g_pool_mu;
+cudaMemPool_t g_pool[kPoolDevices] = {};
+}  // namespace
+
+cudaError_t scratch_alloc(void **p, size_t bytes, cudaStream_t stream) {
+  int dev = 0;
+  cudaError_t e = cudaGetDevice(&dev);
+  if (e != cudaSuccess) return e;
+  if (dev < 0 || dev >= kPoolDevices) return cudaErrorInvalidDevice;
+  cudaMemPool_t pool;
+  {
+    std::lock_guard<std::mutex> lk(g_pool_mu);
+    if (!g_pool[dev]) {
+      cudaMemPoolProps props = {};
+      props.allocType = cudaMemAllocationTypePinned;
+      props.handleTypes = cudaMemHandleTypeNone;
+      props.location.type = cudaMemLocationTypeDevice;
+      props.location.id = dev;
+      cudaMemPool_t np;
+      if ((e = cudaMemPoolCreate(&np, &props)) != cudaSuccess) return e;
+      uint64_t keep = ~0ull;
+      if ((e = cudaMemPoolSetAttribute(np, cudaMemPoolAttrReleaseThreshold, &keep)) != cudaSuccess) return e;
+      g_pool[dev] = np;
+    }
+    pool = g_pool[dev];
+  }
+  return cudaMallocFromPoolAsync(p, bytes, pool, stream);
+}
+
+cudaError_t scratch_trim() {
+  int dev = 0;
+  cudaError_t e = cudaGetDevice(&dev);
+  if (e != cudaSuccess) return e;
+  if (dev < 0 || dev >= kPoolDevices) return cudaErrorInvalidDevice;
+  std::lock_guard<std::mutex> lk(g_pool_mu);
+  return g_pool[dev] ? cudaMemPoolTrimTo(g_pool[dev], 0) : cudaSuccess;
+}
+
 }  // namespace c2d
 
 namespace {
@@ -169,7 +212,9 @@ const char *conv2d_strerror(int code) {
   }
 }
 
-int conv2d_version(void) { return 100; }
+int conv2d_version(void) { return 101; }
+
+int conv2d_release_scratch(void) { return scratch_trim() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA; }
 
 // Not part of include/conv2d.h: selects a kernel variant for tuning tools (0 = default).
 int c2d_debug_set_variant(int v) {

@@ -9,6 +9,7 @@
 #include <cuda_runtime.h>
 
 #include "../../include/conv2d.h"
+#include "common.h"
 
 namespace {
 
@@ -63,7 +64,7 @@ extern "C" int conv2d_single_host(const float *in, int H, int W, const float *fi
 
   void *d_buf = nullptr;
   const size_t in_pad = (in_b + 255) / 256 * 256, out_pad = (out_b + 255) / 256 * 256;
-  if (cudaMallocAsync(&d_buf, in_pad + out_pad + f_b, p.s_in) != cudaSuccess) return CONV2D_EALLOC;
+  if (c2d::scratch_alloc(&d_buf, in_pad + out_pad + f_b, p.s_in) != cudaSuccess) return CONV2D_EALLOC;
   float *d_in = static_cast<float *>(d_buf);
   float *d_out = reinterpret_cast<float *>(static_cast<char *>(d_buf) + in_pad);
   float *d_f = reinterpret_cast<float *>(static_cast<char *>(d_buf) + in_pad + out_pad);

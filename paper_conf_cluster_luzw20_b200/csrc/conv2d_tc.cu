@@ -1,39 +1,69 @@
 // conv2d_tc.cu -- tensor-core variant of the multi-channel convolution: the large-C
-// case is a dense contraction, D[p][f] = sum_k A[p][k] * B[k][f] with p = (n, y, x) output pixels,
-// f filters and k = (c, i, j), A[p][k] = in[n][c][y+i][x+j] (implicit im2col), B[k][f] = w[f][c][i][j].
+// case is a dense contraction, D[p][f] = sum_k A[p][k] * B[k][f] with p output pixels, f filters and
+// k = (c, i, j), A[p][k] = in[n][c][y+i][x+j] (implicit im2col), B[k][f] = w[f][c][i][j].
 // It runs on the 5th-generation tensor cores (tcgen05.mma kind::tf32, accumulator in TMEM) with the
-// 3xTF32 split a = a_hi + a_lo (a_hi = tf32(a), a_lo = a - a_hi exact in fp32):
+// 3xTF32 split a = a_hi + a_lo (a_hi = tf32(a) rounded to nearest, a_lo = a - a_hi exact in fp32):
 //     D = A_hi B_hi + A_hi B_lo + A_lo B_hi      (the dropped A_lo B_lo term is ~2^-22 |a||b|)
 // which keeps each product within ~2^-21 relative, far inside the 1e-5 * sum|x||w| acceptance
 // (DESIGN.md "Tensor-core variant"). A separate, measured variant, as BASELINE.json north_star asks.
 //
-// CTA = 128 threads, one 128-pixel x FN-filter output tile (FN <= 256, TMEM columns = FN), K in blocks
-// of 32. Per K block every thread gathers its pixel's 32 im2col values (coalesced across the warp),
-// splits them and writes A_hi / A_lo into shared memory in the canonical K-major no-swizzle UMMA layout
-// (8-row x 16-byte core matrices); the filter block is split the same way into B_hi / B_lo. Two
-// stages: while the tensor core runs block b, the threads stage block b+1. One elected thread issues
-// 4 x 3 MMAs per block and commits them to the stage's mbarrier. The epilogue reads the accumulator
-// with tcgen05.ld (each warp its 32 TMEM lanes) and stores NFHoWo rows (coalesced along pixels).
+// Design (v2):
+//   * Pixels are indexed with the INPUT row pitch, p = y*W + x (x < W, not Wo): for a fixed
+//     k = (c, i, j) the A column of 128 consecutive pixels is then 128 consecutive input floats at
+//     plane offset p0 + i*W + j, so every gather is one coalesced 128-byte warp load. The W-Wo pixels
+//     per row with x >= Wo are computed from clamped addresses and never stored.
+//   * A (im2col) goes straight from registers to TMEM (tcgen05.st), never through shared memory:
+//     a gather thread owns one pixel row = one TMEM lane, splits its 16 k-values of a K block into
+//     hi/lo and stores them into the 32 + 32 TMEM columns of an A stage; the MMA reads A from
+//     TMEM ("TS" form) and only B from shared memory. This removes the A shared-memory round trip and
+//     the A re-reads that made the first version shared-memory bound.
+//   * B (filters) is split once per call by a small kernel into hi/lo tiles laid out exactly as the
+//     canonical K-major no-swizzle UMMA shared-memory image of each (filter block, K block); a
+//     producer thread streams them with 1-D bulk copies (cp.async.bulk, mbarrier complete_tx) into a
+//     deeper ring than A, so B latency is off the critical path.
+//   * Warp roles (320 threads): warps 0-7 gather A and run the epilogue (warps w and w+4 share TMEM
+//     lane quarter w%4 and take one half of each K block's 32 k), warp 8 allocates TMEM and one lane
+//     issues the MMAs (12 per K block: 4 k-steps x 3 split products) and commits them to the stage
+//     "empty" barriers, warp 9 lane 0 produces B. Global loads of K blocks kb+1 and kb+2 are in
+//     flight in registers while block kb is split and stored.
+//   * Epilogue: tcgen05.ld (each warp its 32 TMEM lanes) -> NFHoWo stores, coalesced along pixels.
 #include <cstdint>
 
 #include <cuda_runtime.h>
 
 #include "../../include/conv2d.h"
+#include "common.h"
 
 namespace c2d_tc {
 
-constexpr int kM = 128;     // pixels per tile (UMMA M)
-constexpr int kKB = 32;     // k values per block (4 UMMA K=8 steps)
-constexpr int kThreads = 256;  // 2 threads per pixel row: each stages 16 of a block's 32 k
+constexpr int kM = 128;        // pixels per tile (UMMA M, TMEM lanes)
+constexpr int kKB = 32;        // k values per K block (4 UMMA K=8 steps)
+constexpr int kGather = 256;   // gather / epilogue threads (warps 0-7: two per TMEM lane quarter)
+constexpr int kMmaWarp = 8;    // TMEM allocation + MMA issue
+constexpr int kProdWarp = 9;   // B producer
+constexpr int kThreads = 320;
+constexpr int kKH = kKB / 2;   // k values per gather thread and K block
 
 __device__ __forceinline__ uint32_t smem_u32(const void *p) {
   return static_cast<uint32_t>(__cvta_generic_to_shared(p));
+}
+
+__host__ __device__ constexpr int tile_elem(int rows, int r, int k) {
+  // element (row r, k) of a [rows x 32] K-major no-swizzle tile: core matrix (k/4, r/8) of 8 rows x 16 B
+  return ((k >> 2) * (rows >> 3) + (r >> 3)) * 32 + (r & 7) * 4 + (k & 3);
 }
 
 __device__ __forceinline__ float tf32_hi(float a) {
   uint32_t r;
   asm("cvt.rna.tf32.f32 %0, %1;" : "=r"(r) : "f"(a));
   return __uint_as_float(r);
+}
+
+// round-to-nearest (ties away) to the tf32 grid on the bit pattern: 2 integer ops instead of the
+// Inf/NaN-guarded cvt.rna sequence. Equal to cvt.rna.tf32 for every finite |a| < 0x1.ffep127 and for
+// +-Inf / NaN (the carry never leaves the exponent field there).
+__device__ __forceinline__ float tf32_hi_fast(float a) {
+  return __uint_as_float((__float_as_uint(a) + 0x1000u) & 0xffffe000u);
 }
 
 // canonical K-major, SWIZZLE_NONE UMMA shared-memory descriptor (cute::UMMA::SmemDescriptor layout):
@@ -54,13 +84,14 @@ __host__ __device__ constexpr uint32_t idesc_tf32(int M, int N) {
          (static_cast<uint32_t>(M >> 4) << 24);
 }
 
-__device__ __forceinline__ void mma_tf32(uint32_t tmem_d, uint64_t adesc, uint64_t bdesc, uint32_t idesc,
-                                         uint32_t accumulate) {
+// D (TMEM) (+)= A (TMEM) x B (shared memory descriptor)
+__device__ __forceinline__ void mma_tf32_ts(uint32_t tmem_d, uint32_t tmem_a, uint64_t bdesc, uint32_t idesc,
+                                            uint32_t accumulate) {
   asm volatile(
       "{\n\t.reg .pred p;\n\t"
       "setp.ne.b32 p, %4, 0;\n\t"
-      "tcgen05.mma.cta_group::1.kind::tf32 [%0], %1, %2, %3, p;\n\t}\n" ::"r"(tmem_d),
-      "l"(adesc), "l"(bdesc), "r"(idesc), "r"(accumulate));
+      "tcgen05.mma.cta_group::1.kind::tf32 [%0], [%1], %2, %3, p;\n\t}\n" ::"r"(tmem_d),
+      "r"(tmem_a), "l"(bdesc), "r"(idesc), "r"(accumulate));
 }
 
 __device__ __forceinline__ void mma_commit(uint32_t mbar) {
@@ -70,6 +101,14 @@ __device__ __forceinline__ void mma_commit(uint32_t mbar) {
 
 __device__ __forceinline__ void mbar_init(uint32_t mbar, uint32_t count) {
   asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(mbar), "r"(count) : "memory");
+}
+
+__device__ __forceinline__ void mbar_arrive(uint32_t mbar) {
+  asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(mbar) : "memory");
+}
+
+__device__ __forceinline__ void mbar_arrive_tx(uint32_t mbar, uint32_t bytes) {
+  asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(mbar), "r"(bytes) : "memory");
 }
 
 __device__ __forceinline__ void mbar_wait(uint32_t mbar, uint32_t parity) {
@@ -82,9 +121,34 @@ __device__ __forceinline__ void mbar_wait(uint32_t mbar, uint32_t parity) {
       : "memory");
 }
 
-__device__ __forceinline__ void fence_async_smem() { asm volatile("fence.proxy.async.shared::cta;" ::: "memory"); }
+__device__ __forceinline__ void bulk_g2s(uint32_t dst, const void *src, uint32_t bytes, uint32_t mbar) {
+  asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(dst),
+               "l"(src), "r"(bytes), "r"(mbar)
+               : "memory");
+}
+
 __device__ __forceinline__ void tc_fence_before() { asm volatile("tcgen05.fence::before_thread_sync;" ::: "memory"); }
 __device__ __forceinline__ void tc_fence_after() { asm volatile("tcgen05.fence::after_thread_sync;" ::: "memory"); }
+
+__device__ __forceinline__ void tmem_st32(uint32_t taddr, const uint32_t (&r)[32]) {
+  asm volatile(
+      "tcgen05.st.sync.aligned.32x32b.x32.b32 [%0], {%1,%2,%3,%4,%5,%6,%7,%8,%9,%10,%11,%12,%13,%14,%15,%16,"
+      "%17,%18,%19,%20,%21,%22,%23,%24,%25,%26,%27,%28,%29,%30,%31,%32};" ::"r"(taddr),
+      "r"(r[0]), "r"(r[1]), "r"(r[2]), "r"(r[3]), "r"(r[4]), "r"(r[5]), "r"(r[6]), "r"(r[7]), "r"(r[8]), "r"(r[9]),
+      "r"(r[10]), "r"(r[11]), "r"(r[12]), "r"(r[13]), "r"(r[14]), "r"(r[15]), "r"(r[16]), "r"(r[17]), "r"(r[18]),
+      "r"(r[19]), "r"(r[20]), "r"(r[21]), "r"(r[22]), "r"(r[23]), "r"(r[24]), "r"(r[25]), "r"(r[26]), "r"(r[27]),
+      "r"(r[28]), "r"(r[29]), "r"(r[30]), "r"(r[31])
+      : "memory");
+}
+
+__device__ __forceinline__ void tmem_st16(uint32_t taddr, const uint32_t (&r)[16]) {
+  asm volatile(
+      "tcgen05.st.sync.aligned.32x32b.x16.b32 [%0], {%1,%2,%3,%4,%5,%6,%7,%8,%9,%10,%11,%12,%13,%14,%15,%16};" ::"r"(
+          taddr),
+      "r"(r[0]), "r"(r[1]), "r"(r[2]), "r"(r[3]), "r"(r[4]), "r"(r[5]), "r"(r[6]), "r"(r[7]), "r"(r[8]), "r"(r[9]),
+      "r"(r[10]), "r"(r[11]), "r"(r[12]), "r"(r[13]), "r"(r[14]), "r"(r[15])
+      : "memory");
+}
 
 __device__ __forceinline__ void tmem_ld16(uint32_t taddr, float (&v)[16]) {
   uint32_t r[16];
@@ -98,194 +162,237 @@ __device__ __forceinline__ void tmem_ld16(uint32_t taddr, float (&v)[16]) {
   for (int i = 0; i < 16; ++i) v[i] = __uint_as_float(r[i]);
 }
 
-struct TcArgs {
-  const float *in;
-  const float *filt;
-  float *out;
-  int N, C, H, W, F, K, Ho, Wo;
-  long long P;   // N * Ho * Wo output pixels
-  int Kg;        // C * K * K
-  int n_kb;      // K blocks
-  int f0;        // first filter of this launch's N tile
-};
-
-// stage bytes: A_hi, A_lo (128 x 32 fp32 each) + B_hi, B_lo (FN x 32 each)
-template <int FN>
-struct Stage {
-  static constexpr uint32_t kA = kM * kKB * 4;   // 16 KiB
-  static constexpr uint32_t kB = FN * kKB * 4;
-  static constexpr uint32_t kBytes = 2 * kA + 2 * kB;
-};
-
-// element (row r, k) of a [rows x 32] K-major no-swizzle tile: core matrix (r/8, k/4) of 8 x 16 B
-__device__ __forceinline__ uint32_t tile_off(int rows, int r, int k) {
-  return static_cast<uint32_t>(((k >> 2) * (rows >> 3) + (r >> 3)) * 128 + (r & 7) * 16 + (k & 3) * 4);
+// ------------------------------------------------------------------------------------------------
+// filter split: Bs[fb][kb] = { hi tile [FN x 32], lo tile [FN x 32] } in the UMMA shared-memory image
+// ------------------------------------------------------------------------------------------------
+__global__ void k_tc_split_filters(const float *__restrict__ filt, int F, int Kg, int FN, int n_kb, int n_fb,
+                                   float *__restrict__ bs) {
+  const long long total = static_cast<long long>(n_fb) * n_kb * FN * kKB;
+  for (long long e = static_cast<long long>(blockIdx.x) * blockDim.x + threadIdx.x; e < total;
+       e += static_cast<long long>(gridDim.x) * blockDim.x) {
+    const int k = static_cast<int>(e % kKB);
+    const int f = static_cast<int>((e / kKB) % FN);
+    const int kb = static_cast<int>((e / (kKB * FN)) % n_kb);
+    const int fb = static_cast<int>(e / (static_cast<long long>(kKB) * FN * n_kb));
+    const int fg = fb * FN + f, kg = kb * kKB + k;
+    const float v = (fg < F && kg < Kg) ? filt[static_cast<size_t>(fg) * Kg + kg] : 0.f;
+    const float hi = tf32_hi(v);
+    float *tile = bs + (static_cast<size_t>(fb) * n_kb + kb) * 2 * FN * kKB;
+    tile[tile_elem(FN, f, k)] = hi;
+    tile[FN * kKB + tile_elem(FN, f, k)] = v - hi;
+  }
 }
 
+// ------------------------------------------------------------------------------------------------
+// main kernel
+// ------------------------------------------------------------------------------------------------
+struct TcArgs {
+  const float *in;
+  const float *bs;  // split filters (k_tc_split_filters)
+  float *out;
+  int N, C, H, W, F, K, Ho, Wo;
+  int Kg;             // C * K * K
+  int n_kb;           // K blocks of 32
+  int tiles_per_img;  // ceil(Ho * W / 128)
+};
+
 template <int FN>
-__global__ void __launch_bounds__(kThreads) k_conv2d_multi_tc3(const TcArgs a) {
-  extern __shared__ __align__(1024) uint8_t smem[];  // [2 stages][A_hi A_lo B_hi B_lo] + int koff[Kg]
-  __shared__ __align__(8) uint64_t mbar[2];
+struct TcCfg {
+  static constexpr int NSA = (FN <= 64) ? 3 : (FN <= 128 ? 2 : 4);  // A stages (TMEM, 64 columns each)
+  static constexpr uint32_t kBStage = 2u * FN * kKB * 4u;            // B hi + lo tile bytes
+  static constexpr int NSB = (FN <= 32) ? 8 : (FN <= 64 ? 6 : 3);    // B stages (shared memory)
+  static constexpr int kCols = FN + NSA * 2 * kKB;                   // TMEM columns used
+  static constexpr int kAlloc = kCols <= 32 ? 32 : kCols <= 64 ? 64 : kCols <= 128 ? 128 : kCols <= 256 ? 256 : 512;
+};
+
+template <int FN, int D>
+__global__ void __launch_bounds__(kThreads, 2) k_conv2d_multi_tc4(const TcArgs a) {
+  using Cfg = TcCfg<FN>;
+  constexpr int NSA = Cfg::NSA, NSB = Cfg::NSB;
+  extern __shared__ __align__(1024) uint8_t smem[];  // [NSB B stages] + int koff[n_kb * 32]
+  __shared__ __align__(8) uint64_t full_a[NSA], empty_a[NSA], full_b[NSB], empty_b[NSB], acc_full;
   __shared__ uint32_t tmem_base_s;
-  constexpr uint32_t SB = Stage<FN>::kBytes;
-  const uint32_t sbase = smem_u32(smem);
   const int tid = threadIdx.x;
   const int warp = tid >> 5;
+  const int lane = tid & 31;
+  int *koff = reinterpret_cast<int *>(smem + NSB * Cfg::kBStage);
 
-  if (warp == 0) {  // TMEM accumulator: FN columns (power of two >= 32)
+  if (warp == kMmaWarp) {  // TMEM: accumulator [0, FN) + NSA A stages of 64 columns
     asm volatile("tcgen05.alloc.cta_group::1.sync.aligned.shared::cta.b32 [%0], %1;" ::"r"(smem_u32(&tmem_base_s)),
-                 "r"(FN));
+                 "r"(Cfg::kAlloc));
     asm volatile("tcgen05.relinquish_alloc_permit.cta_group::1.sync.aligned;");
   }
   if (tid == 0) {
-    mbar_init(smem_u32(&mbar[0]), 1);
-    mbar_init(smem_u32(&mbar[1]), 1);
+    for (int s = 0; s < NSA; ++s) {
+      mbar_init(smem_u32(&full_a[s]), kGather);
+      mbar_init(smem_u32(&empty_a[s]), 1);
+    }
+    for (int s = 0; s < NSB; ++s) {
+      mbar_init(smem_u32(&full_b[s]), 1);
+      mbar_init(smem_u32(&empty_b[s]), 1);
+    }
+    mbar_init(smem_u32(&acc_full), 1);
     asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
   }
+  // im2col offsets of every k = (c, i, j) relative to the pixel's (c=0, y, x) input element; the
+  // padding k >= Kg point at offset 0 (always in range; their B entries are zero)
+  const int KK0 = a.K * a.K;
+  const int plane = a.H * a.W;
+  for (int k = tid; k < a.n_kb * kKB; k += kThreads) {
+    int o = 0;
+    if (k < a.Kg) {
+      const int c = k / KK0, ij = k - c * KK0;
+      const int i = ij / a.K, j = ij - i * a.K;
+      o = c * plane + i * a.W + j;
+    }
+    koff[k] = o;
+  }
   tc_fence_before();
   __syncthreads();
   tc_fence_after();
-  const uint32_t tmem_d = tmem_base_s;
+  const uint32_t tmem = tmem_base_s;
+  const int n = blockIdx.x / a.tiles_per_img;
+  const int t = blockIdx.x - n * a.tiles_per_img;
+  const int fblk = blockIdx.y;
+  const uint32_t sb_base = smem_u32(smem);
 
-  // im2col offsets of every k = (c, i, j) relative to the pixel's (c=0, y, x) input element
-  int *koff = reinterpret_cast<int *>(smem + 2 * SB);
-  for (int k = tid; k < a.Kg; k += kThreads) {
-    const int KK0 = a.K * a.K;
-    const int c = k / KK0, ij = k - c * KK0;
-    const int i = ij / a.K, j = ij - i * a.K;
-    koff[k] = (c * a.H + i) * a.W + j;
-  }
-  __syncthreads();
-  // this thread's pixel (row of A) and half of each K block
-  const int row = tid & (kM - 1);
-  const int khalf = tid / kM;  // 0 or 1: k in [16*khalf, 16*khalf+16) of each block
-  const long long g = static_cast<long long>(blockIdx.x) * kM + row;
-  const bool valid = g < a.P;
-  const long long gg = valid ? g : a.P - 1;
-  const int PP = a.Ho * a.Wo;
-  const int n = static_cast<int>(gg / PP);
-  const int p = static_cast<int>(gg % PP);
-  const int y = p / a.Wo, x = p % a.Wo;
-  const float *__restrict__ pix = a.in + (static_cast<size_t>(n) * a.C * a.H + y) * a.W + x;
-  constexpr uint32_t idesc = idesc_tf32(kM, FN);
+  if (warp < 8) {
+    // ---------------- gather: pixel p = y*W + x of image n ----------------
+    // warp w serves TMEM lane quarter w%4 (pixel rows 32(w%4)..+31) and k half w/4 of every K block
+    const int quarter = warp & 3, khalf = warp >> 2;
+    const int row = quarter * 32 + lane;
+    const int pp = t * kM + row;
+    const int y = pp / a.W, x = pp - y * a.W;
+    const bool valid = (y < a.Ho) && (x < a.Wo);
+    const int pe = valid ? pp : 0;  // garbage pixels read pixel 0's window (in range)
+    const float *__restrict__ img = a.in + static_cast<size_t>(n) * a.C * plane + pe;
+    const uint32_t t_lane = static_cast<uint32_t>(quarter * 32) << 16;
 
-  // gather + split one K block into stage s
-  auto stage_block = [&](int kb, int s) {
-    const uint32_t st = sbase + s * SB;
-    const int k0 = kb * kKB;
-    // A: 16 values of this thread's im2col row (its half of the block), 4 at a time -> one 16-byte
-    // store per (hi, lo); consecutive lanes = consecutive pixels, so each load is coalesced
+    auto load = [&](float (&v)[kKH], int kb) {
+      const int4 *ko = reinterpret_cast<const int4 *>(koff + kb * kKB + khalf * kKH);
 #pragma unroll
-    for (int q = 0; q < kKB / 8; ++q) {
-      const int kq = 16 * khalf + 4 * q;
-      float hi[4], lo[4];
-#pragma unroll
-      for (int t = 0; t < 4; ++t) {
-        const int k = k0 + kq + t;
-        const float v = (k < a.Kg) ? __ldg(pix + koff[k]) : 0.f;
-        hi[t] = tf32_hi(v);
-        lo[t] = v - hi[t];
+      for (int q = 0; q < kKH / 4; ++q) {
+        const int4 o = ko[q];
+        v[4 * q + 0] = __ldg(img + o.x);
+        v[4 * q + 1] = __ldg(img + o.y);
+        v[4 * q + 2] = __ldg(img + o.z);
+        v[4 * q + 3] = __ldg(img + o.w);
       }
-      const uint32_t off = tile_off(kM, row, kq);
-      asm volatile("st.shared.v4.f32 [%0], {%1, %2, %3, %4};" ::"r"(st + off), "f"(hi[0]), "f"(hi[1]), "f"(hi[2]),
-                   "f"(hi[3]) : "memory");
-      asm volatile("st.shared.v4.f32 [%0], {%1, %2, %3, %4};" ::"r"(st + Stage<FN>::kA + off), "f"(lo[0]),
-                   "f"(lo[1]), "f"(lo[2]), "f"(lo[3]) : "memory");
-    }
-    // B: FN filter rows x 32 k (contiguous in FCKK), 4 at a time
-    for (int e = tid; e < FN * (kKB / 4); e += kThreads) {
-      const int f = e / (kKB / 4), q = e % (kKB / 4);
-      const int fg = a.f0 + f;
-      float hi[4], lo[4];
-#pragma unroll
-      for (int t = 0; t < 4; ++t) {
-        const int k = k0 + 4 * q + t;
-        const float v = (fg < a.F && k < a.Kg) ? __ldg(a.filt + static_cast<size_t>(fg) * a.Kg + k) : 0.f;
-        hi[t] = tf32_hi(v);
-        lo[t] = v - hi[t];
+    };
+    auto put = [&](float (&v)[kKH], int kb) {
+      const int s = kb % NSA;
+      if (kb >= NSA) {
+        mbar_wait(smem_u32(&empty_a[s]), static_cast<uint32_t>((kb / NSA - 1) & 1));
+        tc_fence_after();
       }
-      const uint32_t off = tile_off(FN, f, 4 * q);
-      asm volatile("st.shared.v4.f32 [%0], {%1, %2, %3, %4};" ::"r"(st + 2 * Stage<FN>::kA + off), "f"(hi[0]),
-                   "f"(hi[1]), "f"(hi[2]), "f"(hi[3]) : "memory");
-      asm volatile("st.shared.v4.f32 [%0], {%1, %2, %3, %4};" ::"r"(st + 2 * Stage<FN>::kA + Stage<FN>::kB + off),
-                   "f"(lo[0]), "f"(lo[1]), "f"(lo[2]), "f"(lo[3]) : "memory");
-    }
-    fence_async_smem();  // generic-proxy smem writes -> visible to the tensor core (async proxy)
-  };
-
-  auto issue_block = [&](int kb, int s) {
-    const uint32_t st = sbase + s * SB;
-    const uint32_t a_hi = st, a_lo = st + Stage<FN>::kA;
-    const uint32_t b_hi = st + 2 * Stage<FN>::kA, b_lo = b_hi + Stage<FN>::kB;
+      if (kb == a.n_kb - 1) {  // padding k >= Kg: exact zeros (no Inf/NaN from the clamped reads)
 #pragma unroll
-    for (int kk = 0; kk < kKB / 8; ++kk) {
-      // K = 8 tf32 = two 16-byte chunks: chunk (2kk) and (2kk+1) of the tile
-      const uint32_t ao = static_cast<uint32_t>(2 * kk * (kM / 8) * 128);
-      const uint32_t bo = static_cast<uint32_t>(2 * kk * (FN / 8) * 128);
-      const uint32_t a_lbo = (kM / 8) * 128, b_lbo = (FN / 8) * 128;
-      const uint64_t dah = umma_desc(a_hi + ao, a_lbo, 128), dal = umma_desc(a_lo + ao, a_lbo, 128);
-      const uint64_t dbh = umma_desc(b_hi + bo, b_lbo, 128), dbl = umma_desc(b_lo + bo, b_lbo, 128);
-      const uint32_t acc0 = (kb > 0 || kk > 0) ? 1u : 0u;
-      mma_tf32(tmem_d, dah, dbh, idesc, acc0);
-      mma_tf32(tmem_d, dah, dbl, idesc, 1u);
-      mma_tf32(tmem_d, dal, dbh, idesc, 1u);
-    }
-    mma_commit(smem_u32(&mbar[s]));
-  };
-
-  // two-stage pipeline: stage kb+1 while the tensor core runs kb
-  uint32_t phase[2] = {0u, 0u};
-  stage_block(0, 0);
-  __syncthreads();
-  for (int kb = 0; kb < a.n_kb; ++kb) {
-    const int s = kb & 1;
-    if (tid == 0) {
-      tc_fence_after();
-      issue_block(kb, s);
-    }
-    if (kb + 1 < a.n_kb) {
-      const int s2 = s ^ 1;
-      if (kb >= 1) {  // stage s2 was consumed by the MMAs of block kb-1
-        mbar_wait(smem_u32(&mbar[s2]), phase[s2]);
-        phase[s2] ^= 1u;
+        for (int q = 0; q < kKH; ++q)
+          if (kb * kKB + khalf * kKH + q >= a.Kg) v[q] = 0.f;
       }
-      stage_block(kb + 1, s2);
+      uint32_t hi[kKH], lo[kKH];
+#pragma unroll
+      for (int q = 0; q < kKH; ++q) {
+        const float h = tf32_hi_fast(v[q]);
+        hi[q] = __float_as_uint(h);
+        lo[q] = __float_as_uint(v[q] - h);
+      }
+      const uint32_t col = tmem + t_lane + FN + s * 2 * kKB + khalf * kKH;
+      tmem_st16(col, hi);
+      tmem_st16(col + kKB, lo);
+      asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory");
+      tc_fence_before();
+      mbar_arrive(smem_u32(&full_a[s]));
+    };
+    // ring of D register buffers: the loads of K blocks kb+1 .. kb+D-1 are in flight while block kb
+    // is split and stored
+    float v[D][kKH];
+#pragma unroll
+    for (int d = 0; d < D; ++d)
+      if (d < a.n_kb) load(v[d], d);
+    for (int kb0 = 0; kb0 < a.n_kb; kb0 += D) {
+#pragma unroll
+      for (int d = 0; d < D; ++d) {
+        const int kb = kb0 + d;
+        if (kb < a.n_kb) {
+          put(v[d], kb);
+          if (kb + D < a.n_kb) load(v[d], kb + D);
+        }
+      }
     }
-    __syncthreads();
-  }
-  // the last block's commit tracks every MMA issued before it: its completion means D is final
-  // (every earlier commit of that stage was waited on above, so phase[] is current)
-  {
-    const int s_last = (a.n_kb - 1) & 1;
-    mbar_wait(smem_u32(&mbar[s_last]), phase[s_last]);
-  }
-  tc_fence_after();
 
-  // epilogue: TMEM -> registers -> out[n][f][p]. Warp w may only access TMEM lanes 32(w%4)..+31, so
-  // warps w and w+4 split the accumulator columns of the same 32 pixels.
-  const uint32_t lane_base = static_cast<uint32_t>((warp & 3) * 32) << 16;
+    // ---------------- epilogue: TMEM accumulator -> out[n][f][y][x] ----------------
+    mbar_wait(smem_u32(&acc_full), 0);
+    tc_fence_after();
+    const size_t PP = static_cast<size_t>(a.Ho) * a.Wo;
+    float *__restrict__ obase = a.out + (static_cast<size_t>(n) * a.F) * PP + (valid ? (y * a.Wo + x) : 0);
+    const int f0 = fblk * FN;
 #pragma unroll 1
-  for (int c0 = 16 * khalf; c0 < FN; c0 += 32) {
-    float v[16];
-    tmem_ld16(tmem_d + lane_base + c0, v);
-    if (valid) {
+    for (int c0 = khalf * (FN / 2); c0 < (khalf + 1) * (FN / 2); c0 += 16) {
+      float v[16];
+      tmem_ld16(tmem + t_lane + c0, v);
+      if (valid) {
 #pragma unroll
-      for (int t = 0; t < 16; ++t) {
-        const int f = a.f0 + c0 + t;
-        if (f < a.F) a.out[(static_cast<size_t>(n) * a.F + f) * PP + p] = v[t];
+        for (int q = 0; q < 16; ++q) {
+          const int f = f0 + c0 + q;
+          if (f < a.F) __stcs(obase + static_cast<size_t>(f) * PP, v[q]);
+        }
+      }
+    }
+  } else if (warp == kMmaWarp) {
+    // ---------------- MMA issuer ----------------
+    if (lane == 0) {
+      constexpr uint32_t idesc = idesc_tf32(kM, FN);
+      constexpr uint32_t lbo = (FN / 8) * 128;
+      for (int kb = 0; kb < a.n_kb; ++kb) {
+        const int sa = kb % NSA, sb = kb % NSB;
+        mbar_wait(smem_u32(&full_a[sa]), static_cast<uint32_t>((kb / NSA) & 1));
+        mbar_wait(smem_u32(&full_b[sb]), static_cast<uint32_t>((kb / NSB) & 1));
+        tc_fence_after();
+        const uint32_t a_hi = tmem + FN + sa * 2 * kKB, a_lo = a_hi + kKB;
+        const uint32_t b_hi = sb_base + sb * Cfg::kBStage, b_lo = b_hi + Cfg::kBStage / 2;
+#pragma unroll
+        for (int kk = 0; kk < kKB / 8; ++kk) {
+          const uint32_t bo = static_cast<uint32_t>(2 * kk * (FN / 8) * 128);
+          const uint64_t dbh = umma_desc(b_hi + bo, lbo, 128), dbl = umma_desc(b_lo + bo, lbo, 128);
+          const uint32_t acc0 = (kb > 0 || kk > 0) ? 1u : 0u;
+          mma_tf32_ts(tmem, a_hi + 8 * kk, dbh, idesc, acc0);
+          mma_tf32_ts(tmem, a_hi + 8 * kk, dbl, idesc, 1u);
+          mma_tf32_ts(tmem, a_lo + 8 * kk, dbh, idesc, 1u);
+        }
+        mma_commit(smem_u32(&empty_a[sa]));
+        mma_commit(smem_u32(&empty_b[sb]));
+      }
+      mma_commit(smem_u32(&acc_full));
+    }
+  } else {
+    // ---------------- B producer: bulk copies of the split filter tiles ----------------
+    if (lane == 0) {
+      const float *src = a.bs + static_cast<size_t>(fblk) * a.n_kb * (Cfg::kBStage / 4);
+      for (int kb = 0; kb < a.n_kb; ++kb) {
+        const int sb = kb % NSB;
+        if (kb >= NSB) mbar_wait(smem_u32(&empty_b[sb]), static_cast<uint32_t>((kb / NSB - 1) & 1));
+        mbar_arrive_tx(smem_u32(&full_b[sb]), Cfg::kBStage);
+        bulk_g2s(sb_base + sb * Cfg::kBStage, src + static_cast<size_t>(kb) * (Cfg::kBStage / 4), Cfg::kBStage,
+                 smem_u32(&full_b[sb]));
       }
     }
   }
   tc_fence_before();
   __syncthreads();
-  if (warp == 0)
-    asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem_d), "r"(FN));
+  if (warp == kMmaWarp) {
+    tc_fence_after();
+    asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"(Cfg::kAlloc));
+  }
 }
 
-template <int FN>
-int launch_tc(const TcArgs &a0, cudaStream_t stream) {
-  auto kernel = k_conv2d_multi_tc3<FN>;
-  const size_t smem = 2 * Stage<FN>::kBytes + static_cast<size_t>(a0.Kg) * sizeof(int);
+// Split the filters into a stream-ordered scratch buffer, run the main kernel over (pixel tiles x
+// filter blocks), free the scratch (stream-ordered).
+template <int FN, int D>
+int launch_tc_d(TcArgs a, const float *filt, cudaStream_t stream) {
+  using Cfg = TcCfg<FN>;
+  auto kernel = k_conv2d_multi_tc4<FN, D>;
+  const size_t smem = static_cast<size_t>(Cfg::NSB) * Cfg::kBStage + static_cast<size_t>(a.n_kb) * kKB * sizeof(int);
   static int max_dyn = 0;  // dynamic shared memory enabled for this instantiation
   if (max_dyn == 0) {
     int dev = 0, optin = 0;
@@ -304,14 +411,37 @@ int launch_tc(const TcArgs &a0, cudaStream_t stream) {
     max_dyn = avail;
   }
   if (smem > static_cast<size_t>(max_dyn)) return CONV2D_ESHAPE;
-  TcArgs a = a0;
-  const long long blocks = (a.P + kM - 1) / kM;
-  for (int f0 = 0; f0 < a.F; f0 += FN) {
-    a.f0 = f0;
-    kernel<<<static_cast<unsigned>(blocks), kThreads, smem, stream>>>(a);
-    if (cudaGetLastError() != cudaSuccess) return CONV2D_ECUDA;
+  const int n_fb = (a.F + FN - 1) / FN;
+  const size_t bs_bytes = static_cast<size_t>(n_fb) * a.n_kb * Cfg::kBStage;
+  float *bs = nullptr;
+  if (c2d::scratch_alloc(reinterpret_cast<void **>(&bs), bs_bytes, stream) != cudaSuccess) {
+    (void)cudaGetLastError();
+    return CONV2D_EALLOC;
   }
-  return CONV2D_OK;
+  int rc = CONV2D_OK;
+  const long long split_elems = static_cast<long long>(n_fb) * a.n_kb * FN * kKB;
+  const int split_blocks = static_cast<int>(split_elems / 256 < 1184 ? (split_elems + 255) / 256 : 1184);
+  k_tc_split_filters<<<split_blocks, 256, 0, stream>>>(filt, a.F, a.Kg, FN, a.n_kb, n_fb, bs);
+  if (cudaGetLastError() != cudaSuccess) rc = CONV2D_ECUDA;
+  if (rc == CONV2D_OK) {
+    a.bs = bs;
+    const dim3 grid(static_cast<unsigned>(static_cast<long long>(a.N) * a.tiles_per_img), static_cast<unsigned>(n_fb));
+    kernel<<<grid, kThreads, smem, stream>>>(a);
+    if (cudaGetLastError() != cudaSuccess) rc = CONV2D_ECUDA;
+  }
+  if (cudaFreeAsync(bs, stream) != cudaSuccess && rc == CONV2D_OK) rc = CONV2D_ECUDA;
+  return rc;
+}
+
+// register ring depth D (K blocks per gather thread in registers): 2 by default (measured on B200:
+// configs[2] 98 vs 96 / 93 TFLOP/s for D = 3 / 4, which spill at the 96-register cap of two CTAs
+// per SM); the multi-channel tuning override (c2d_debug_set_multi_variant) 23 / 24 selects 3 / 4
+template <int FN>
+int launch_tc(const TcArgs &a, const float *filt, cudaStream_t stream) {
+  const int mv = c2d::g_mvariant.load(std::memory_order_relaxed);
+  if (mv == 23) return launch_tc_d<FN, 3>(a, filt, stream);
+  if (mv == 24) return launch_tc_d<FN, 4>(a, filt, stream);
+  return launch_tc_d<FN, 2>(a, filt, stream);
 }
 
 }  // namespace c2d_tc
@@ -325,9 +455,12 @@ extern "C" int conv2d_multi_tc(const float *in, int N, int C, int H, int W, cons
   if (N < 1 || C < 1 || F < 1 || H < K || W < K) return CONV2D_ESHAPE;
   if ((reinterpret_cast<uintptr_t>(in) | reinterpret_cast<uintptr_t>(filt) | reinterpret_cast<uintptr_t>(out)) & 3u)
     return CONV2D_EALIGN;
+  // 32-bit in-image offsets (one image's C planes) and a bounded im2col offset table
+  if (static_cast<long long>(C) * H * W >= (1LL << 31) || static_cast<long long>(C) * K * K > (1 << 14))
+    return CONV2D_ESHAPE;
   TcArgs a;
   a.in = in;
-  a.filt = filt;
+  a.bs = nullptr;
   a.out = out;
   a.N = N;
   a.C = C;
@@ -337,15 +470,17 @@ extern "C" int conv2d_multi_tc(const float *in, int N, int C, int H, int W, cons
   a.K = K;
   a.Ho = H - K + 1;
   a.Wo = W - K + 1;
-  a.P = static_cast<long long>(N) * a.Ho * a.Wo;
   a.Kg = C * K * K;
   a.n_kb = (a.Kg + kKB - 1) / kKB;
-  a.f0 = 0;
-  const double px = static_cast<double>(a.P);
-  if (px / kM > 2147483647.0) return CONV2D_ESHAPE;
+  a.tiles_per_img = static_cast<int>((static_cast<long long>(a.Ho) * W + kM - 1) / kM);
+  if (static_cast<long long>(N) * a.tiles_per_img > 2147483647LL) return CONV2D_ESHAPE;
   cudaStream_t s = static_cast<cudaStream_t>(stream);
-  if (F <= 32) return launch_tc<32>(a, s);
-  if (F <= 64) return launch_tc<64>(a, s);
-  if (F <= 128) return launch_tc<128>(a, s);
-  return launch_tc<256>(a, s);
+  // filter block FN = the smallest of 32/64/128/256 covering F; a smaller block when the larger one's
+  // shared memory (B ring + offset table) does not fit
+  int rc = CONV2D_ESHAPE;
+  if (F > 128) rc = launch_tc<256>(a, filt, s);
+  if (rc == CONV2D_ESHAPE && F > 64) rc = launch_tc<128>(a, filt, s);
+  if (rc == CONV2D_ESHAPE && F > 32) rc = launch_tc<64>(a, filt, s);
+  if (rc == CONV2D_ESHAPE) rc = launch_tc<32>(a, filt, s);
+  return rc;
 }

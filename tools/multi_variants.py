@@ -56,10 +56,11 @@ def main():
         ref = None
         line = f"{name:32s}"
         for vs in a.variants.split(","):
-            v = -1 if vs == "tc" else int(vs)
+            # "tc" = tensor-core variant (default tuning), "tcNN" = with multi variant override NN
+            v = -1 if vs.startswith("tc") else int(vs)
             fn = (lambda out=None: pkg.conv2d_multi_tc(x, w, out=out)) if v < 0 else \
                 (lambda out=None: pkg.conv2d_multi(x, w, out=out))
-            _capi.debug_set_multi_variant(max(v, 0))
+            _capi.debug_set_multi_variant(int(vs[2:] or 0) if v < 0 else v)
             try:
                 y = fn()
                 torch.cuda.synchronize()
@@ -72,7 +73,7 @@ def main():
             ms = time_call(lambda: fn(out=y))
             if v < 0:  # the tensor-core variant is not bitwise equal: report its max relative deviation
                 dev = float(((y - ref).abs().max() / ref.abs().max().clamp_min(1e-30)).item())
-                line += f"  tc {flops / ms / 1e9:6.1f} TF (max dev {dev:.1e})"
+                line += f"  {vs} {flops / ms / 1e9:6.1f} TF (max dev {dev:.1e})"
             else:
                 line += f"  v{v} {flops / ms / 1e9:6.1f} TF{'' if same else ' DIFF'}"
         _capi.debug_set_multi_variant(0)

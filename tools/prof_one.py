@@ -28,6 +28,7 @@ def main():
     ap.add_argument("--time", action="store_true")
     ap.add_argument("--variant", type=int, default=0)
     ap.add_argument("--mvariant", type=int, default=0)
+    ap.add_argument("--tc", action="store_true", help="multi: the tensor-core variant conv2d_multi_tc")
     a = ap.parse_args()
     pkg._capi.debug_set_variant(a.variant)
     pkg._capi.debug_set_multi_variant(a.mvariant)
@@ -44,7 +45,7 @@ def main():
         N, C, H, W, F = [int(v) for v in a.shape.split(",")]
         x = synth.fill_torch(1, 1, (N, C, H, W), "img", device=dev)
         w = torch.from_numpy(synth.make_filter(1, a.K, "he", F=F, C=C)).to(dev)
-        fn = lambda: pkg.conv2d_multi(x, w, band_h=a.band)  # noqa: E731
+        fn = (lambda: pkg.conv2d_multi_tc(x, w)) if a.tc else (lambda: pkg.conv2d_multi(x, w, band_h=a.band))
         work = 2.0 * N * F * (H - a.K + 1) * (W - a.K + 1) * C * a.K * a.K
     for _ in range(a.reps):
         fn()
