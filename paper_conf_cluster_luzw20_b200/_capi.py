@@ -36,7 +36,7 @@ def load(path: str | None = None):
     global _lib
     if _lib is not None:
         return _lib
-    p = path or LIB_PATH
+    p = path or os.environ.get("C2D_LIB") or LIB_PATH  # C2D_LIB: tuning builds (tools/) only
     if not os.path.exists(p):
         raise ImportError(f"{p} is missing: run `python -c 'import __graft_entry__ as g; g.build()'` "
                           "(there is no fallback implementation)")

@@ -150,6 +150,22 @@ __device__ __forceinline__ void tmem_st16(uint32_t taddr, const uint32_t (&r)[16
       : "memory");
 }
 
+__device__ __forceinline__ void tmem_st8(uint32_t taddr, const uint32_t (&r)[8]) {
+  asm volatile("tcgen05.st.sync.aligned.32x32b.x8.b32 [%0], {%1,%2,%3,%4,%5,%6,%7,%8};" ::"r"(taddr), "r"(r[0]),
+               "r"(r[1]), "r"(r[2]), "r"(r[3]), "r"(r[4]), "r"(r[5]), "r"(r[6]), "r"(r[7])
+               : "memory");
+}
+
+template <int NV>
+__device__ __forceinline__ void tmem_stv(uint32_t taddr, const uint32_t (&r)[NV]) {
+  if constexpr (NV == 16) {
+    tmem_st16(taddr, r);
+  } else {
+    static_assert(NV == 8, "8 or 16 columns");
+    tmem_st8(taddr, r);
+  }
+}
+
 __device__ __forceinline__ void tmem_ld16(uint32_t taddr, float (&v)[16]) {
   uint32_t r[16];
   asm volatile(
@@ -196,18 +212,23 @@ struct TcArgs {
   int tiles_per_img;  // ceil(Ho * W / 128)
 };
 
-template <int FN>
+// NBS: B ring depth selector (0 = default; otherwise the stage count, for tuning)
+// NACC: 1 = one accumulator; 2 = A_hi B_hi into accumulator 0 and the two correction products into
+// accumulator 1 (summed in the epilogue) -- two independent MMA dependency chains per CTA
+template <int FN, int NBS = 0, int NACC = 1>
 struct TcCfg {
-  static constexpr int NSA = (FN <= 64) ? 3 : (FN <= 128 ? 2 : 4);  // A stages (TMEM, 64 columns each)
+  static constexpr int NSA = NACC == 1 ? ((FN <= 64) ? 3 : (FN <= 128 ? 2 : 4))
+                                       : ((FN <= 32) ? 3 : (FN <= 64 ? 2 : 4));  // A stages (TMEM, 64 cols)
   static constexpr uint32_t kBStage = 2u * FN * kKB * 4u;            // B hi + lo tile bytes
-  static constexpr int NSB = (FN <= 32) ? 8 : (FN <= 64 ? 6 : 3);    // B stages (shared memory)
-  static constexpr int kCols = FN + NSA * 2 * kKB;                   // TMEM columns used
+  static constexpr int NSB = NBS ? NBS : ((FN <= 32) ? 8 : (FN <= 64 ? 6 : 3));  // B stages (smem)
+  static constexpr int kAcc = NACC * FN;
+  static constexpr int kCols = kAcc + NSA * 2 * kKB;                 // TMEM columns used
   static constexpr int kAlloc = kCols <= 32 ? 32 : kCols <= 64 ? 64 : kCols <= 128 ? 128 : kCols <= 256 ? 256 : 512;
 };
 
-template <int FN, int D>
+template <int FN, int D, int NBS, int NACC>
 __global__ void __launch_bounds__(kThreads, 2) k_conv2d_multi_tc4(const TcArgs a) {
-  using Cfg = TcCfg<FN>;
+  using Cfg = TcCfg<FN, NBS, NACC>;
   constexpr int NSA = Cfg::NSA, NSB = Cfg::NSB;
   extern __shared__ __align__(1024) uint8_t smem[];  // [NSB B stages] + int koff[n_kb * 32]
   __shared__ __align__(8) uint64_t full_a[NSA], empty_a[NSA], full_b[NSB], empty_b[NSB], acc_full;
@@ -297,7 +318,7 @@ __global__ void __launch_bounds__(kThreads, 2) k_conv2d_multi_tc4(const TcArgs a
         hi[q] = __float_as_uint(h);
         lo[q] = __float_as_uint(v[q] - h);
       }
-      const uint32_t col = tmem + t_lane + FN + s * 2 * kKB + khalf * kKH;
+      const uint32_t col = tmem + t_lane + Cfg::kAcc + s * 2 * kKB + khalf * kKH;
       tmem_st16(col, hi);
       tmem_st16(col + kKB, lo);
       asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory");
@@ -331,6 +352,12 @@ __global__ void __launch_bounds__(kThreads, 2) k_conv2d_multi_tc4(const TcArgs a
     for (int c0 = khalf * (FN / 2); c0 < (khalf + 1) * (FN / 2); c0 += 16) {
       float v[16];
       tmem_ld16(tmem + t_lane + c0, v);
+      if constexpr (NACC == 2) {
+        float c[16];
+        tmem_ld16(tmem + t_lane + FN + c0, c);
+#pragma unroll
+        for (int q = 0; q < 16; ++q) v[q] += c[q];
+      }
       if (valid) {
 #pragma unroll
         for (int q = 0; q < 16; ++q) {
@@ -349,16 +376,17 @@ __global__ void __launch_bounds__(kThreads, 2) k_conv2d_multi_tc4(const TcArgs a
         mbar_wait(smem_u32(&full_a[sa]), static_cast<uint32_t>((kb / NSA) & 1));
         mbar_wait(smem_u32(&full_b[sb]), static_cast<uint32_t>((kb / NSB) & 1));
         tc_fence_after();
-        const uint32_t a_hi = tmem + FN + sa * 2 * kKB, a_lo = a_hi + kKB;
+        const uint32_t a_hi = tmem + Cfg::kAcc + sa * 2 * kKB, a_lo = a_hi + kKB;
         const uint32_t b_hi = sb_base + sb * Cfg::kBStage, b_lo = b_hi + Cfg::kBStage / 2;
+        const uint32_t d1 = tmem + (NACC == 2 ? FN : 0);  // accumulator of the correction products
 #pragma unroll
         for (int kk = 0; kk < kKB / 8; ++kk) {
           const uint32_t bo = static_cast<uint32_t>(2 * kk * (FN / 8) * 128);
           const uint64_t dbh = umma_desc(b_hi + bo, lbo, 128), dbl = umma_desc(b_lo + bo, lbo, 128);
           const uint32_t acc0 = (kb > 0 || kk > 0) ? 1u : 0u;
           mma_tf32_ts(tmem, a_hi + 8 * kk, dbh, idesc, acc0);
-          mma_tf32_ts(tmem, a_hi + 8 * kk, dbl, idesc, 1u);
-          mma_tf32_ts(tmem, a_lo + 8 * kk, dbh, idesc, 1u);
+          mma_tf32_ts(d1, a_hi + 8 * kk, dbl, idesc, NACC == 2 ? acc0 : 1u);
+          mma_tf32_ts(d1, a_lo + 8 * kk, dbh, idesc, 1u);
         }
         mma_commit(smem_u32(&empty_a[sa]));
         mma_commit(smem_u32(&empty_b[sb]));
@@ -386,33 +414,296 @@ __global__ void __launch_bounds__(kThreads, 2) k_conv2d_multi_tc4(const TcArgs a
   }
 }
 
-// Split the filters into a stream-ordered scratch buffer, run the main kernel over (pixel tiles x
-// filter blocks), free the scratch (stream-ordered).
-template <int FN, int D>
-int launch_tc_d(TcArgs a, const float *filt, cudaStream_t stream) {
-  using Cfg = TcCfg<FN>;
-  auto kernel = k_conv2d_multi_tc4<FN, D>;
-  const size_t smem = static_cast<size_t>(Cfg::NSB) * Cfg::kBStage + static_cast<size_t>(a.n_kb) * kKB * sizeof(int);
-  static int max_dyn = 0;  // dynamic shared memory enabled for this instantiation
-  if (max_dyn == 0) {
-    int dev = 0, optin = 0;
-    cudaFuncAttributes fa;
-    if (cudaGetDevice(&dev) != cudaSuccess ||
-        cudaDeviceGetAttribute(&optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev) != cudaSuccess ||
-        cudaFuncGetAttributes(&fa, kernel) != cudaSuccess) {
-      (void)cudaGetLastError();
-      return CONV2D_ECUDA;
-    }
-    const int avail = optin - static_cast<int>(fa.sharedSizeBytes);
-    if (cudaFuncSetAttribute(kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, avail) != cudaSuccess) {
-      (void)cudaGetLastError();
-      return CONV2D_ECUDA;
-    }
-    max_dyn = avail;
+// ------------------------------------------------------------------------------------------------
+// persistent kernel: one CTA per SM walks the tiles (pixel tile x filter block) of the launch; two
+// TMEM accumulators let the epilogue of tile j run on dedicated warps while the MMAs of tile j+1
+// accumulate into the other buffer, and the A / B rings run continuously across tile boundaries
+// ------------------------------------------------------------------------------------------------
+// warps [0, GW): A gather (GW/4 per TMEM lane quarter, each a 32*4/GW-wide k slice of every K
+// block); [GW, GW+4): epilogue; GW+4: TMEM allocation + MMA issue; GW+5: B producer
+template <int GW>
+struct TcPWarps {
+  static constexpr int kGather = GW * 32;
+  static constexpr int kEpi0 = GW;
+  static constexpr int kMma = GW + 4;
+  static constexpr int kProd = GW + 5;
+  static constexpr int kThreads = (GW + 6) * 32;
+  static constexpr int kKS = kKB * 4 / GW;  // k values per gather thread and K block
+};
+
+template <int FN>
+struct TcPCfg {
+  static constexpr int NSA = 4;                          // A stages (TMEM, 64 columns each)
+  static constexpr uint32_t kBStage = 2u * FN * kKB * 4u;  // B hi + lo tile bytes
+  static constexpr int NSB = (FN <= 64) ? 8 : 4;         // B stages (shared memory, 128 KB)
+  static constexpr int kAcc = 2 * FN;                    // two accumulators
+  static constexpr int kCols = kAcc + NSA * 2 * kKB;
+  static_assert(kCols <= 512, "TMEM");
+  static constexpr int kAlloc = kCols <= 256 ? 256 : 512;
+};
+
+struct TcTile {
+  int n, t, fblk;
+};
+
+__device__ __forceinline__ TcTile tc_tile(const TcArgs &a, int n_fb, int tile) {
+  TcTile r;
+  const int pt = tile / n_fb;  // filter blocks innermost: consecutive tiles share their pixels
+  r.fblk = tile - pt * n_fb;
+  r.n = pt / a.tiles_per_img;
+  r.t = pt - r.n * a.tiles_per_img;
+  return r;
+}
+
+template <int FN, int D, int GW>
+__global__ void __launch_bounds__(TcPWarps<GW>::kThreads, 1) k_conv2d_multi_tc5(const TcArgs a, int n_fb, int n_tiles) {
+  using Cfg = TcPCfg<FN>;
+  using Wp = TcPWarps<GW>;
+  constexpr int KS = Wp::kKS;
+  constexpr int NSA = Cfg::NSA, NSB = Cfg::NSB;
+  extern __shared__ __align__(1024) uint8_t smem[];  // [NSB B stages] + int koff[n_kb * 32]
+  __shared__ __align__(8) uint64_t full_a[NSA], empty_a[NSA], full_b[NSB], empty_b[NSB], acc_full[2],
+      acc_empty[2];
+  __shared__ uint32_t tmem_base_s;
+  const int tid = threadIdx.x;
+  const int warp = tid >> 5;
+  const int lane = tid & 31;
+  int *koff = reinterpret_cast<int *>(smem + NSB * Cfg::kBStage);
+
+  if (warp == Wp::kMma) {
+    asm volatile("tcgen05.alloc.cta_group::1.sync.aligned.shared::cta.b32 [%0], %1;" ::"r"(smem_u32(&tmem_base_s)),
+                 "r"(Cfg::kAlloc));
+    asm volatile("tcgen05.relinquish_alloc_permit.cta_group::1.sync.aligned;");
   }
-  if (smem > static_cast<size_t>(max_dyn)) return CONV2D_ESHAPE;
+  if (tid == 0) {
+    for (int s = 0; s < NSA; ++s) {
+      mbar_init(smem_u32(&full_a[s]), Wp::kGather);
+      mbar_init(smem_u32(&empty_a[s]), 1);
+    }
+    for (int s = 0; s < NSB; ++s) {
+      mbar_init(smem_u32(&full_b[s]), 1);
+      mbar_init(smem_u32(&empty_b[s]), 1);
+    }
+    for (int b = 0; b < 2; ++b) {
+      mbar_init(smem_u32(&acc_full[b]), 1);
+      mbar_init(smem_u32(&acc_empty[b]), 128);
+    }
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+  }
+  const int KK0 = a.K * a.K;
+  const int plane = a.H * a.W;
+  for (int k = tid; k < a.n_kb * kKB; k += Wp::kThreads) {
+    int o = 0;
+    if (k < a.Kg) {
+      const int c = k / KK0, ij = k - c * KK0;
+      const int i = ij / a.K, j = ij - i * a.K;
+      o = c * plane + i * a.W + j;
+    }
+    koff[k] = o;
+  }
+  tc_fence_before();
+  __syncthreads();
+  tc_fence_after();
+  const uint32_t tmem = tmem_base_s;
+  const uint32_t sb_base = smem_u32(smem);
+  // this CTA's tiles: blockIdx.x, blockIdx.x + gridDim.x, ...; local block stream g = j * n_kb + kb
+  const int my_tiles = (n_tiles - static_cast<int>(blockIdx.x) + static_cast<int>(gridDim.x) - 1) /
+                       static_cast<int>(gridDim.x);
+  const int n_blocks = my_tiles * a.n_kb;
+  // small filter banks (one filter block, K blocks <= ring stages) are loaded once and stay resident
+  const bool b_resident = (n_fb == 1) && (a.n_kb <= NSB);
+
+  if (warp < GW) {
+    // ---------------- gather (A producer) ----------------
+    const int quarter = warp & 3, kpart = warp >> 2;
+    const int row = quarter * 32 + lane;
+    const uint32_t t_lane = static_cast<uint32_t>(quarter * 32) << 16;
+    // pixel base pointer of local tile j (garbage pixels read pixel 0's in-range window)
+    auto tile_img = [&](int j) -> const float * {
+      const TcTile tt = tc_tile(a, n_fb, static_cast<int>(blockIdx.x) + j * static_cast<int>(gridDim.x));
+      const int pp = tt.t * kM + row;
+      const int y = pp / a.W, x = pp - y * a.W;
+      const int pe = (y < a.Ho && x < a.Wo) ? pp : 0;
+      return a.in + static_cast<size_t>(tt.n) * a.C * plane + pe;
+    };
+    auto load = [&](float (&v)[KS], int g) {
+      const int j = g / a.n_kb, kb = g - j * a.n_kb;
+      const float *__restrict__ img = tile_img(j);
+      const int4 *ko = reinterpret_cast<const int4 *>(koff + kb * kKB + kpart * KS);
+#pragma unroll
+      for (int q = 0; q < KS / 4; ++q) {
+        const int4 o = ko[q];
+        v[4 * q + 0] = __ldg(img + o.x);
+        v[4 * q + 1] = __ldg(img + o.y);
+        v[4 * q + 2] = __ldg(img + o.z);
+        v[4 * q + 3] = __ldg(img + o.w);
+      }
+    };
+    auto put = [&](float (&v)[KS], int g) {
+      const int s = g % NSA;
+      if (g >= NSA) {
+        mbar_wait(smem_u32(&empty_a[s]), static_cast<uint32_t>((g / NSA - 1) & 1));
+        tc_fence_after();
+      }
+      const int kb = g % a.n_kb;
+      if (kb == a.n_kb - 1) {  // padding k >= Kg: exact zeros
+#pragma unroll
+        for (int q = 0; q < KS; ++q)
+          if (kb * kKB + kpart * KS + q >= a.Kg) v[q] = 0.f;
+      }
+      uint32_t hi[KS], lo[KS];
+#pragma unroll
+      for (int q = 0; q < KS; ++q) {
+        const float h = tf32_hi_fast(v[q]);
+        hi[q] = __float_as_uint(h);
+        lo[q] = __float_as_uint(v[q] - h);
+      }
+      const uint32_t col = tmem + t_lane + Cfg::kAcc + s * 2 * kKB + kpart * KS;
+      tmem_stv<KS>(col, hi);
+      tmem_stv<KS>(col + kKB, lo);
+      asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory");
+      tc_fence_before();
+      mbar_arrive(smem_u32(&full_a[s]));
+    };
+    // ring of D register buffers: blocks g+1 .. g+D-1 in flight while block g is split and stored
+    float v[D][KS];
+#pragma unroll
+    for (int d = 0; d < D; ++d)
+      if (d < n_blocks) load(v[d], d);
+    for (int g0 = 0; g0 < n_blocks; g0 += D) {
+#pragma unroll
+      for (int d = 0; d < D; ++d) {
+        const int g = g0 + d;
+        if (g < n_blocks) {
+          put(v[d], g);
+          if (g + D < n_blocks) load(v[d], g + D);
+        }
+      }
+    }
+  } else if (warp < GW + 4) {
+    // ---------------- epilogue: TMEM accumulator -> out[n][f][y][x] ----------------
+    const int quarter = warp & 3;
+    const int row = quarter * 32 + lane;
+    const uint32_t t_lane = static_cast<uint32_t>(quarter * 32) << 16;
+    const size_t PP = static_cast<size_t>(a.Ho) * a.Wo;
+    for (int j = 0; j < my_tiles; ++j) {
+      const int ab = j & 1;
+      const TcTile tt = tc_tile(a, n_fb, static_cast<int>(blockIdx.x) + j * static_cast<int>(gridDim.x));
+      const int pp = tt.t * kM + row;
+      const int y = pp / a.W, x = pp - y * a.W;
+      const bool valid = (y < a.Ho) && (x < a.Wo);
+      float *__restrict__ obase = a.out + (static_cast<size_t>(tt.n) * a.F) * PP + (valid ? (y * a.Wo + x) : 0);
+      const int f0 = tt.fblk * FN;
+      mbar_wait(smem_u32(&acc_full[ab]), static_cast<uint32_t>((j >> 1) & 1));
+      tc_fence_after();
+#pragma unroll 1
+      for (int c0 = 0; c0 < FN; c0 += 16) {
+        float v[16];
+        tmem_ld16(tmem + t_lane + ab * FN + c0, v);
+        if (valid) {
+#pragma unroll
+          for (int q = 0; q < 16; ++q) {
+            const int f = f0 + c0 + q;
+            if (f < a.F) __stcs(obase + static_cast<size_t>(f) * PP, v[q]);
+          }
+        }
+      }
+      tc_fence_before();
+      mbar_arrive(smem_u32(&acc_empty[ab]));
+    }
+  } else if (warp == Wp::kMma) {
+    // ---------------- MMA issuer ----------------
+    if (lane == 0) {
+      constexpr uint32_t idesc = idesc_tf32(kM, FN);
+      constexpr uint32_t lbo = (FN / 8) * 128;
+      int g = 0;
+      for (int j = 0; j < my_tiles; ++j) {
+        const int ab = j & 1;
+        if (j >= 2) {  // the epilogue of tile j-2 has drained this accumulator
+          mbar_wait(smem_u32(&acc_empty[ab]), static_cast<uint32_t>(((j >> 1) - 1) & 1));
+          tc_fence_after();
+        }
+        const uint32_t d = tmem + ab * FN;
+        for (int kb = 0; kb < a.n_kb; ++kb, ++g) {
+          const int sa = g % NSA, sb = b_resident ? kb : g % NSB;
+          mbar_wait(smem_u32(&full_a[sa]), static_cast<uint32_t>((g / NSA) & 1));
+          mbar_wait(smem_u32(&full_b[sb]), b_resident ? 0u : static_cast<uint32_t>((g / NSB) & 1));
+          tc_fence_after();
+          const uint32_t a_hi = tmem + Cfg::kAcc + sa * 2 * kKB, a_lo = a_hi + kKB;
+          const uint32_t b_hi = sb_base + sb * Cfg::kBStage, b_lo = b_hi + Cfg::kBStage / 2;
+#pragma unroll
+          for (int kk = 0; kk < kKB / 8; ++kk) {
+            const uint32_t bo = static_cast<uint32_t>(2 * kk * (FN / 8) * 128);
+            const uint64_t dbh = umma_desc(b_hi + bo, lbo, 128), dbl = umma_desc(b_lo + bo, lbo, 128);
+            const uint32_t acc0 = (kb > 0 || kk > 0) ? 1u : 0u;
+            mma_tf32_ts(d, a_hi + 8 * kk, dbh, idesc, acc0);
+            mma_tf32_ts(d, a_hi + 8 * kk, dbl, idesc, 1u);
+            mma_tf32_ts(d, a_lo + 8 * kk, dbh, idesc, 1u);
+          }
+          mma_commit(smem_u32(&empty_a[sa]));
+          if (!b_resident) mma_commit(smem_u32(&empty_b[sb]));
+        }
+        mma_commit(smem_u32(&acc_full[ab]));
+      }
+    }
+  } else {
+    // ---------------- B producer ----------------
+    if (lane == 0 && b_resident) {  // every K block of the one filter block stays in shared memory
+      for (int kb = 0; kb < a.n_kb; ++kb) {
+        mbar_arrive_tx(smem_u32(&full_b[kb]), Cfg::kBStage);
+        bulk_g2s(sb_base + kb * Cfg::kBStage, a.bs + static_cast<size_t>(kb) * (Cfg::kBStage / 4), Cfg::kBStage,
+                 smem_u32(&full_b[kb]));
+      }
+    } else if (lane == 0) {
+      int g = 0;
+      for (int j = 0; j < my_tiles; ++j) {
+        const TcTile tt = tc_tile(a, n_fb, static_cast<int>(blockIdx.x) + j * static_cast<int>(gridDim.x));
+        const float *src = a.bs + static_cast<size_t>(tt.fblk) * a.n_kb * (Cfg::kBStage / 4);
+        for (int kb = 0; kb < a.n_kb; ++kb, ++g) {
+          const int sb = g % NSB;
+          if (g >= NSB) mbar_wait(smem_u32(&empty_b[sb]), static_cast<uint32_t>((g / NSB - 1) & 1));
+          mbar_arrive_tx(smem_u32(&full_b[sb]), Cfg::kBStage);
+          bulk_g2s(sb_base + sb * Cfg::kBStage, src + static_cast<size_t>(kb) * (Cfg::kBStage / 4), Cfg::kBStage,
+                   smem_u32(&full_b[sb]));
+        }
+      }
+    }
+  }
+  tc_fence_before();
+  __syncthreads();
+  if (warp == Wp::kMma) {
+    tc_fence_after();
+    asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"(Cfg::kAlloc));
+  }
+}
+
+// Enable the dynamic shared memory a kernel instantiation may use (once per instantiation).
+template <typename KernelT>
+int enable_smem(KernelT kernel, int &max_dyn) {
+  if (max_dyn > 0) return CONV2D_OK;
+  int dev = 0, optin = 0;
+  cudaFuncAttributes fa;
+  if (cudaGetDevice(&dev) != cudaSuccess ||
+      cudaDeviceGetAttribute(&optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev) != cudaSuccess ||
+      cudaFuncGetAttributes(&fa, kernel) != cudaSuccess) {
+    (void)cudaGetLastError();
+    return CONV2D_ECUDA;
+  }
+  const int avail = optin - static_cast<int>(fa.sharedSizeBytes);
+  if (cudaFuncSetAttribute(kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, avail) != cudaSuccess) {
+    (void)cudaGetLastError();
+    return CONV2D_ECUDA;
+  }
+  max_dyn = avail;
+  return CONV2D_OK;
+}
+
+// Split the filters into a stream-ordered scratch buffer from the library pool, run `body(bs, n_fb)`
+// (the main kernel launch), free the scratch (stream-ordered).
+template <int FN, typename Body>
+int with_split_filters(const TcArgs &a, const float *filt, cudaStream_t stream, Body body) {
   const int n_fb = (a.F + FN - 1) / FN;
-  const size_t bs_bytes = static_cast<size_t>(n_fb) * a.n_kb * Cfg::kBStage;
+  const size_t bs_bytes = static_cast<size_t>(n_fb) * a.n_kb * (2u * FN * kKB * 4u);
   float *bs = nullptr;
   if (c2d::scratch_alloc(reinterpret_cast<void **>(&bs), bs_bytes, stream) != cudaSuccess) {
     (void)cudaGetLastError();
@@ -423,25 +714,71 @@ int launch_tc_d(TcArgs a, const float *filt, cudaStream_t stream) {
   const int split_blocks = static_cast<int>(split_elems / 256 < 1184 ? (split_elems + 255) / 256 : 1184);
   k_tc_split_filters<<<split_blocks, 256, 0, stream>>>(filt, a.F, a.Kg, FN, a.n_kb, n_fb, bs);
   if (cudaGetLastError() != cudaSuccess) rc = CONV2D_ECUDA;
-  if (rc == CONV2D_OK) {
-    a.bs = bs;
-    const dim3 grid(static_cast<unsigned>(static_cast<long long>(a.N) * a.tiles_per_img), static_cast<unsigned>(n_fb));
-    kernel<<<grid, kThreads, smem, stream>>>(a);
-    if (cudaGetLastError() != cudaSuccess) rc = CONV2D_ECUDA;
-  }
+  if (rc == CONV2D_OK) rc = body(bs, n_fb);
   if (cudaFreeAsync(bs, stream) != cudaSuccess && rc == CONV2D_OK) rc = CONV2D_ECUDA;
   return rc;
 }
 
-// register ring depth D (K blocks per gather thread in registers): 2 by default (measured on B200:
-// configs[2] 98 vs 96 / 93 TFLOP/s for D = 3 / 4, which spill at the 96-register cap of two CTAs
-// per SM); the multi-channel tuning override (c2d_debug_set_multi_variant) 23 / 24 selects 3 / 4
+// one CTA per (pixel tile, filter block), two CTAs per SM
+template <int FN, int D, int NBS = 0, int NACC = 1>
+int launch_tc_d(TcArgs a, const float *filt, cudaStream_t stream) {
+  using Cfg = TcCfg<FN, NBS, NACC>;
+  auto kernel = k_conv2d_multi_tc4<FN, D, NBS, NACC>;
+  const size_t smem = static_cast<size_t>(Cfg::NSB) * Cfg::kBStage + static_cast<size_t>(a.n_kb) * kKB * sizeof(int);
+  static int max_dyn = 0;
+  if (enable_smem(kernel, max_dyn) != CONV2D_OK) return CONV2D_ECUDA;
+  if (smem > static_cast<size_t>(max_dyn)) return CONV2D_ESHAPE;
+  return with_split_filters<FN>(a, filt, stream, [&](const float *bs, int n_fb) {
+    a.bs = bs;
+    const dim3 grid(static_cast<unsigned>(static_cast<long long>(a.N) * a.tiles_per_img), static_cast<unsigned>(n_fb));
+    kernel<<<grid, kThreads, smem, stream>>>(a);
+    return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
+  });
+}
+
+// persistent: one CTA per SM over all (pixel tile, filter block) tiles
+template <int FN, int D, int GW>
+int launch_tc_p(TcArgs a, const float *filt, cudaStream_t stream) {
+  using Cfg = TcPCfg<FN>;
+  auto kernel = k_conv2d_multi_tc5<FN, D, GW>;
+  const size_t smem = static_cast<size_t>(Cfg::NSB) * Cfg::kBStage + static_cast<size_t>(a.n_kb) * kKB * sizeof(int);
+  static int max_dyn = 0;
+  if (enable_smem(kernel, max_dyn) != CONV2D_OK) return CONV2D_ECUDA;
+  if (smem > static_cast<size_t>(max_dyn)) return CONV2D_ESHAPE;
+  int dev = 0, n_sm = 0;
+  if (cudaGetDevice(&dev) != cudaSuccess || cudaDeviceGetAttribute(&n_sm, cudaDevAttrMultiProcessorCount, dev) != cudaSuccess)
+    return CONV2D_ECUDA;
+  return with_split_filters<FN>(a, filt, stream, [&](const float *bs, int n_fb) {
+    a.bs = bs;
+    const long long tiles = static_cast<long long>(a.N) * a.tiles_per_img * n_fb;
+    if (tiles > 2147483647LL) return CONV2D_ESHAPE;
+    const int grid = static_cast<int>(tiles < n_sm ? tiles : n_sm);
+    kernel<<<grid, TcPWarps<GW>::kThreads, smem, stream>>>(a, n_fb, static_cast<int>(tiles));
+    return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
+  });
+}
+
+// Default: the persistent kernel. Tuning overrides (c2d_debug_set_multi_variant): 40 = one CTA per
+// tile (k_conv2d_multi_tc4, register ring depth 2), 23 / 24 = that with depth 3 / 4, 32-34 = with a
+// B ring of 2-4 stages.
 template <int FN>
 int launch_tc(const TcArgs &a, const float *filt, cudaStream_t stream) {
   const int mv = c2d::g_mvariant.load(std::memory_order_relaxed);
+  if (mv == 40) return launch_tc_d<FN, 2, 2>(a, filt, stream);
+  if (mv == 41) return launch_tc_d<FN, 2, 2, 2>(a, filt, stream);
+  if (mv == 42) return launch_tc_d<FN, 2, 3, 2>(a, filt, stream);
   if (mv == 23) return launch_tc_d<FN, 3>(a, filt, stream);
   if (mv == 24) return launch_tc_d<FN, 4>(a, filt, stream);
-  return launch_tc_d<FN, 2>(a, filt, stream);
+  if (mv == 32) return launch_tc_d<FN, 2, 2>(a, filt, stream);
+  if (mv == 33) return launch_tc_d<FN, 2, 3>(a, filt, stream);
+  if (mv == 34) return launch_tc_d<FN, 2, 4>(a, filt, stream);
+  if (mv == 50) return launch_tc_p<FN, 2, 8>(a, filt, stream);
+  if (mv == 51) return launch_tc_p<FN, 3, 8>(a, filt, stream);
+  if (mv == 52) return launch_tc_p<FN, 4, 8>(a, filt, stream);
+  if (mv == 53) return launch_tc_p<FN, 2, 16>(a, filt, stream);
+  if (mv == 54) return launch_tc_p<FN, 3, 16>(a, filt, stream);
+  if (mv == 55) return launch_tc_p<FN, 4, 16>(a, filt, stream);
+  return launch_tc_d<FN, 2, 2>(a, filt, stream);
 }
 
 }  // namespace c2d_tc
@@ -475,11 +812,10 @@ extern "C" int conv2d_multi_tc(const float *in, int N, int C, int H, int W, cons
   a.tiles_per_img = static_cast<int>((static_cast<long long>(a.Ho) * W + kM - 1) / kM);
   if (static_cast<long long>(N) * a.tiles_per_img > 2147483647LL) return CONV2D_ESHAPE;
   cudaStream_t s = static_cast<cudaStream_t>(stream);
-  // filter block FN = the smallest of 32/64/128/256 covering F; a smaller block when the larger one's
-  // shared memory (B ring + offset table) does not fit
+  // filter block FN = the smallest of 32/64/128 covering F (F > 128: several 128-filter blocks); a
+  // smaller block when the larger one's shared memory (B ring + offset table) does not fit
   int rc = CONV2D_ESHAPE;
-  if (F > 128) rc = launch_tc<256>(a, filt, s);
-  if (rc == CONV2D_ESHAPE && F > 64) rc = launch_tc<128>(a, filt, s);
+  if (F > 64) rc = launch_tc<128>(a, filt, s);
   if (rc == CONV2D_ESHAPE && F > 32) rc = launch_tc<64>(a, filt, s);
   if (rc == CONV2D_ESHAPE) rc = launch_tc<32>(a, filt, s);
   return rc;

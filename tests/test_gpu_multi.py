@@ -96,7 +96,9 @@ def test_table1_layers(cuda_device, layer):
 
 
 @pytest.mark.parametrize("shape", [(2, 64, 56, 56, 64, 3), (1, 3, 40, 45, 16, 5), (2, 16, 20, 37, 100, 3),
-                                   (1, 8, 33, 30, 64, 7), (3, 1, 28, 28, 32, 3), (1, 4, 19, 21, 256, 1)])
+                                   (1, 8, 33, 30, 64, 7), (3, 1, 28, 28, 32, 3), (1, 4, 19, 21, 256, 1),
+                                   (1, 3, 7, 7, 300, 7), (2, 2, 9, 130, 129, 2), (40, 3, 30, 33, 40, 3),
+                                   (1, 1, 15, 15, 1, 15)])
 def test_tensor_core_variant(cuda_device, shape):
     """conv2d_multi_tc (tcgen05 3xTF32 implicit GEMM) meets the same 1e-5*sum|x||w| acceptance."""
     N, C, H, W, F, K = shape
@@ -115,3 +117,30 @@ def test_tensor_core_variant_config2_sampled(cuda_device):
     P = 800
     check_points_multi(x, w, y, rng.integers(0, N, P), rng.integers(0, F, P), rng.integers(0, S - K + 1, P),
                        rng.integers(0, S - K + 1, P))
+
+
+@pytest.mark.parametrize("layer", [("CONV1", 28, 128, 3), ("CONV3", 12, 64, 5), ("CONV5", 24, 256, 5),
+                                   ("CONV8", 28, 512, 3), ("CONV11", 224, 64, 3)])
+def test_tensor_core_variant_table1(cuda_device, layer):
+    """PAPER.md Table I layer shapes through the tensor-core variant, C in {1, 3},
+    reduced batch, every output."""
+    name, S, F, K = layer
+    for C in (1, 3):
+        x = dev_image((2, C, S, S), "img", seed=S + C)
+        w = _w(F, C, K, "he", seed=F)
+        check_full_multi(x, w, pkg.conv2d_multi_tc(x, w))
+
+
+def test_tensor_core_variant_config3_sampled(cuda_device):
+    """configs[3] (N=128, C=3, F=64, 224^2, K=7) at full size through the tensor-core variant, sampled
+    outputs (every image, filter and edge row/column appear)."""
+    N, C, F, S, K = 128, 3, 64, 224, 7
+    x = dev_image((N, C, S, S), "img", seed=synth.BASE_SEED + 3)
+    w = _w(F, C, K, "he", seed=synth.BASE_SEED + 3)
+    y = pkg.conv2d_multi_tc(x, w)
+    rng = np.random.default_rng(33)
+    P = 1500
+    Ho = S - K + 1
+    ys = np.concatenate([rng.integers(0, Ho, P), np.array([0, Ho - 1] * 50)])
+    xs = np.concatenate([rng.integers(0, Ho, P), np.array([Ho - 1, 0] * 50)])
+    check_points_multi(x, w, y, rng.integers(0, N, len(ys)), rng.integers(0, F, len(ys)), ys, xs)

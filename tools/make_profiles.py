@@ -26,6 +26,8 @@ CAPTURES = {
     "prof_k15_v0_s8192": "conv2d_single 8192^2 K=15",
     "prof_k3_v0_s8192": "conv2d_single 8192^2 K=3",
     "prof_direct_k3_s8192": "conv2d_single_direct 8192^2 K=3 (Fig. 1a baseline)",
+    "prof_tc_config2": "conv2d_multi_tc N32 C64 F64 56^2 K3",
+    "prof_tc_config3": "conv2d_multi_tc N128 C3 F64 224^2 K7",
 }
 
 
@@ -65,6 +67,16 @@ def main():
         line = open(b).read().strip().splitlines()[-1]
         json.loads(line)
         open(os.path.join(dst, f"{tag}_bench.json"), "w").write(line + "\n")
+    for f in sorted(os.listdir(src)):  # the other workloads' bench lines
+        m = re.fullmatch(rf"bench_{re.escape(tag)}_(\w+)\.json", f)
+        if m:
+            lines = open(os.path.join(src, f)).read().strip().splitlines()
+            if lines:
+                try:
+                    json.loads(lines[-1])
+                except ValueError:
+                    continue
+                open(os.path.join(dst, f"{tag}_bench_{m.group(1)}.json"), "w").write(lines[-1] + "\n")
     lfile = os.path.join(src, f"launches_{tag}.csv")
     if os.path.exists(lfile):
         launches(lfile, os.path.join(dst, f"{tag}_launches.csv"), os.path.join(dst, f"{tag}_launch_shares.txt"))
