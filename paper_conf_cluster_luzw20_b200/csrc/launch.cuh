@@ -13,6 +13,7 @@
 #include "common.h"
 #include "conv2d_kernels.cuh"
 #include "conv2d_multi.cuh"
+#include "conv2d_split.cuh"
 
 namespace {
 
@@ -44,6 +45,8 @@ int cta_occupancy(KernelT kernel, size_t dyn_smem, std::atomic<int> &cache, int 
 // Variant override for tuning tools (c2d_debug_set_variant; 0 = the tuned default):
 //   1: filter in shared memory, U=1 (4 warps/CTA)     2: shared memory, U=2
 //   3: filter in a __constant__ slot, U=1 (1 warp/CTA) 4: __constant__ slot, U=2
+//   5-9: guard / prefetch variants of the constant-slot kernel (see launch_single)
+//   10-12: filter-row split over G parts (conv2d_split.cuh)
 
 // Constant-bank filter slot of this unit (this K), per device: it holds the filter of the last call
 // with this K. A call waits (stream-ordered) for the event recorded behind the previous kernel that
@@ -125,6 +128,83 @@ int launch_single_v(const float *in, int H, int W, const float *filt, float *out
   return go();
 }
 
+// Filter-row split (conv2d_split.cuh): same tile geometry as launch_single_v, but a tile takes G
+// warps -- a cluster of G one-warp CTAs (CL = 1) or one CTA of G warps (CL = 0) -- so a full wave has
+// G times fewer, taller bands.
+template <int K, int G, int U, int PF, int R, int GUARDS, int CL>
+int launch_split_v(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
+                   const DevInfo &dev, int min_band) {
+  static_assert(G >= 1 && G <= 8 && G <= K, "portable cluster of at most K CTAs");
+  auto kernel = k_conv2d_split<K, G, U, PF, R, GUARDS, CL>;
+  static std::atomic<int> occ_cache{0};
+  const size_t smem = static_cast<size_t>(SplitSmem<K, U, PF, R>::kPart) * (CL ? 1 : G);
+  const int threads = CL ? kWarp : G * kWarp;
+  SplitArgs a;
+  a.in = in;
+  a.out = out;
+  a.H = H;
+  a.W = W;
+  a.Ho = H - K + 1;
+  a.Wo = W - K + 1;
+  a.n_cb = ceil_div(a.Wo, 128 * U);
+  a.aligned = (aligned16(in) && (W % 4 == 0)) ? 1 : 0;
+  static std::atomic<int> smem_set{0};
+  if (smem > 48 * 1024 && smem_set.load() == 0) {
+    if (smem > static_cast<size_t>(dev.smem_optin)) return CONV2D_ESHAPE;
+    if (cudaFuncSetAttribute(kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, dev.smem_optin) != cudaSuccess)
+      return CONV2D_ECUDA;
+    smem_set.store(1);
+  }
+  cudaLaunchConfig_t cfg = {};
+  cfg.blockDim = dim3(threads, 1, 1);
+  cfg.dynamicSmemBytes = smem;
+  cfg.stream = stream;
+  cudaLaunchAttribute attr[1];
+  attr[0].id = cudaLaunchAttributeClusterDimension;
+  attr[0].val.clusterDim.x = G;
+  attr[0].val.clusterDim.y = 1;
+  attr[0].val.clusterDim.z = 1;
+  cfg.attrs = attr;
+  cfg.numAttrs = CL ? 1 : 0;
+  if (band_h <= 0) {
+    // resident tiles of one full wave (clusters: as the cluster scheduler places them)
+    int v = occ_cache.load(std::memory_order_relaxed);
+    if (v <= 0) {
+      if constexpr (CL) {
+        cfg.gridDim = dim3(G * dev.num_sms, 1, 1);
+        int clusters = 0;
+        if (cudaOccupancyMaxActiveClusters(&clusters, kernel, &cfg) != cudaSuccess || clusters < 1) clusters = 1;
+        v = clusters;
+      } else {
+        int blocks = 0;
+        if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, kernel, threads, smem) != cudaSuccess ||
+            blocks < 1)
+          blocks = 1;
+        v = blocks * dev.num_sms;
+      }
+      occ_cache.store(v, std::memory_order_relaxed);
+    }
+    const long long bands = v / a.n_cb > 0 ? v / a.n_cb : 1;
+    band_h = ceil_div(a.Ho, bands);
+    if (band_h < min_band) band_h = min_band;
+  }
+  if (band_h > a.Ho) band_h = a.Ho;
+  a.band_h = band_h;
+  const int n_bands = ceil_div(a.Ho, band_h);
+  const long long tiles = static_cast<long long>(a.n_cb) * n_bands;
+  if (tiles * G > 0x7fffffffLL) return CONV2D_ESHAPE;
+  a.n_tiles = static_cast<int>(tiles);
+  cfg.gridDim = dim3(static_cast<unsigned>(CL ? tiles * G : tiles), 1, 1);
+  auto go = [&]() {
+    if (cudaLaunchKernelEx(&cfg, kernel, a) != cudaSuccess) {
+      (void)cudaGetLastError();  // launch-configuration errors are not sticky: do not leak into the next call
+      return CONV2D_ECUDA;
+    }
+    return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
+  };
+  return with_const_filter(filt, K, KCfg<K>::KP, stream, go);
+}
+
 template <int K>
 int launch_single(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
                   const DevInfo &dev) {
@@ -146,6 +226,27 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
     case 9: if (constant_ok) return C2D_LS(1, FSRC_CONST, 4, 2); break;
     default: break;
   }
+  // filter-row split (conv2d_split.cuh; variants 10-12)
+#define C2D_SP(GG, UU, PFF, RR, CLL) \
+  launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(in, H, W, filt, out, stream, band_h, dev, 1)
+  if (constant_ok && v >= 10 && v <= 12) {
+    if constexpr (K >= 3) {
+      switch (v) {
+        case 10: return C2D_SP(2, 1, 4, 4, 1);  // cluster of 2 one-warp CTAs (the default below)
+        case 11: return C2D_SP(2, 1, 4, 8, 0);  // one CTA of 2 warps (same sums: same bits as 10)
+        case 12: return C2D_SP(3, 1, 4, 8, 0);  // one CTA of 3 warps
+        default: break;
+      }
+    }
+  }
+  // Narrow images with large K (latency regime: a full wave of one-warp tiles leaves bands of a few
+  // rows, and the K-1 prologue rows of Alg. 2 case 1 dominate): filter rows split over a cluster of 2
+  // one-warp CTAs (tools/split_sweep.py: 1024^2 K=15 24 -> 30 Gpx/s, 256^2 K=15 1.6 -> 3.8).
+  // Keyed on (W, K) only, so row bands of one image (same W) take the same kernel: bitwise seams.
+  if constexpr (K >= 11) {
+    if (constant_ok && v == 0 && W <= 1024) return C2D_SP(2, 1, 4, 4, 1);
+  }
+#undef C2D_SP
   // Tuned on B200 (tools/variants.py sweeps):
   //   K <= 5        two 128-column chunks per warp; row fetch from a 4-stage cp.async ring, except
   //                 K <= 3 on wide images (one register row in flight is enough when HBM-bound);

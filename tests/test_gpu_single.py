@@ -171,14 +171,16 @@ def test_config4_32768_k15_sampled(cuda_device):
 @pytest.mark.parametrize("variant", [1, 2, 3, 4, 5, 6])
 def test_every_kernel_variant_bitwise_equal(cuda_device, variant):
     """Every instantiation (filter in shared / constant memory, 1 or 2 column chunks, guarded or
-    unguarded band prologue/epilogue) gives the same bits as the default, and passes the oracle."""
+    unguarded band prologue/epilogue) of the one-warp-tile kernel gives the same bits as variant 1,
+    and passes the oracle. (The default takes the filter-row split kernel for W <= 1024, K >= 11;
+    its bits are covered by test_split_variants.)"""
     shapes = [(40, 300), (77, 1030), (300, 517)]
     try:
         for K in (1, 2, 3, 5, 8, 9, 12, 15):
             f = _filt(K, "rand", seed=K)
             for (dh, W) in shapes:
                 x = dev_image((K + dh, W), "img", seed=K * 7 + W)
-                _capi.debug_set_variant(0)
+                _capi.debug_set_variant(1)
                 ref = pkg.conv2d_single(x, f)
                 _capi.debug_set_variant(variant)
                 got = pkg.conv2d_single(x, f)
@@ -188,6 +190,42 @@ def test_every_kernel_variant_bitwise_equal(cuda_device, variant):
                     check_full_single(x, f, got)
                 for bh in (1, 3, K + 1):
                     assert torch.equal(pkg.conv2d_single(x, f, band_h=bh), ref), (variant, K, bh)
+    finally:
+        _capi.debug_set_variant(0)
+
+
+@pytest.mark.parametrize("K", [3, 4, 7, 11, 13, 15])
+def test_split_variants(cuda_device, K):
+    """Filter-row split kernel (conv2d_split.cuh): cluster of 2 one-warp CTAs (variant 10, the default
+    for W <= 1024 and K >= 11), one CTA of 2 warps (11) and of 3 warps (12). Each passes the oracle on
+    ragged / misaligned-pitch shapes, is bitwise band-independent (chunk tails, one-row bands), is
+    exact on integer data, and 10 and 11 (same split, same sums) agree bit for bit."""
+    shapes = [(1, 300), (40, 301), (77, 1030), (300, 517), (9, 129)]
+    f = _filt(K, "rand", seed=K)
+    try:
+        for (dh, W) in shapes:
+            x = dev_image((K + dh, W), "img", seed=K * 11 + W)
+            outs = {}
+            for v in (10, 11, 12):
+                _capi.debug_set_variant(v)
+                y = pkg.conv2d_single(x, f)
+                torch.cuda.synchronize()
+                check_full_single(x, f, y)
+                for bh in (1, 5, 9, K + 2):
+                    assert torch.equal(pkg.conv2d_single(x, f, band_h=bh), y), (v, K, W, bh)
+                outs[v] = y
+            assert torch.equal(outs[10], outs[11]), (K, dh, W)
+            xi = dev_image((K + dh, W), "int", seed=K + W)
+            fi = _filt(K, "int", seed=K)
+            for v in (10, 12):
+                _capi.debug_set_variant(v)
+                check_full_single(xi, fi, pkg.conv2d_single(xi, fi), exact=True)
+        _capi.debug_set_variant(0)
+        if K >= 11:  # the default is variant 10 for narrow images
+            x = dev_image((K + 50, 1000), "img", seed=K)
+            y0 = pkg.conv2d_single(x, f)
+            _capi.debug_set_variant(10)
+            assert torch.equal(pkg.conv2d_single(x, f), y0)
     finally:
         _capi.debug_set_variant(0)
 
