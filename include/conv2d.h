@@ -88,6 +88,23 @@ int conv2d_multi_ex(const float *in, int N, int C, int H, int W, const float *fi
                     float *out, void *stream, int band_h);
 
 /*
+ * Row-band call with a separate halo segment (BASELINE.json north_star "row-band
+ * split ... with a (K-1)-row halo"): the same operation as conv2d_single on an image of
+ * H + halo_rows rows whose first H rows are at `in` and whose last halo_rows rows are at `halo`, both
+ * row-major with pitch W. Output: (H + halo_rows - K + 1) x (W - K + 1), dense row-major at `out`.
+ * The kernels read the halo rows directly from `halo`, which may be another GPU's memory mapped into
+ * this device's address space (CUDA IPC / symmetric memory over NVLink): a rank of a row-band
+ * decomposition then computes its whole band in one launch, reading its neighbour's first K-1 rows
+ * over NVLink, with no exchange step and no tail call. Outputs are bitwise equal to conv2d_single
+ * on the concatenated rows (same kernels, same per-output summation order).
+ * halo_rows == 0 (halo may be NULL) is conv2d_single. Errors as conv2d_single, plus CONV2D_ENULL for
+ * a NULL halo with halo_rows > 0, CONV2D_ESHAPE for halo_rows < 0, and CONV2D_EOVERLAP if `out`
+ * overlaps the halo rows. The halo memory must stay valid and unchanged until the work completes.
+ */
+int conv2d_single_halo(const float *in, int H, int W, const float *halo, int halo_rows, const float *filt,
+                       int K, float *out, void *stream);
+
+/*
  * Baseline "direct convolution" of PAPER.md Fig. 1a: one thread per
  * output element, each thread loads its K*K inputs itself (no column or row reuse). Same arguments,
  * result and error codes as conv2d_single. Kept as the control for the memory-transaction evidence

@@ -4,11 +4,12 @@
 The product is libconv2d.so (C ABI, include/conv2d.h). This package is its thin Python binding:
     _capi   ctypes marshalling of the C entry points (same names)
     api     torch-tensor wrappers (device memory / streams only)
-    shard   multi-GPU partitioning: batch, filter and row-band (with a (K-1)-row NCCL halo)
+    shard   multi-GPU partitioning: batch, filter and row-band (a (K-1)-row halo by NCCL P2P, or read
+            in place from the neighbour's memory over NVLink by conv2d_single_halo)
 """
 from . import _capi
 from .api import (conv2d_multi, conv2d_multi_host, conv2d_multi_tc, conv2d_single, conv2d_single_direct,
-                  conv2d_single_host)
+                  conv2d_single_halo, conv2d_single_host)
 
 __all__ = ["_capi", "conv2d_multi", "conv2d_multi_host", "conv2d_multi_tc", "conv2d_single",
-           "conv2d_single_direct", "conv2d_single_host"]
+           "conv2d_single_direct", "conv2d_single_halo", "conv2d_single_host"]

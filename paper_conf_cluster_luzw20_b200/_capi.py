@@ -9,7 +9,8 @@ _PKG = os.path.dirname(os.path.abspath(__file__))
 LIB_PATH = os.path.join(_PKG, "libconv2d.so")
 
 # every symbol include/conv2d.h declares
-EXPORTS = ("conv2d_single", "conv2d_multi", "conv2d_single_ex", "conv2d_multi_ex", "conv2d_single_direct",
+EXPORTS = ("conv2d_single", "conv2d_multi", "conv2d_single_ex", "conv2d_multi_ex", "conv2d_single_halo",
+           "conv2d_single_direct",
            "conv2d_single_host", "conv2d_multi_tc", "conv2d_release_scratch", "conv2d_strerror", "conv2d_version")
 
 CONV2D_OK = 0
@@ -44,13 +45,14 @@ def load(path: str | None = None):
     P, I = ctypes.c_void_p, ctypes.c_int
     L.conv2d_single.argtypes = [P, I, I, P, I, P, P]
     L.conv2d_single_ex.argtypes = [P, I, I, P, I, P, P, I]
+    L.conv2d_single_halo.argtypes = [P, I, I, P, I, P, I, P, P]
     L.conv2d_single_direct.argtypes = [P, I, I, P, I, P, P]
     L.conv2d_multi.argtypes = [P, I, I, I, I, P, I, I, P, P]
     L.conv2d_multi_ex.argtypes = [P, I, I, I, I, P, I, I, P, P, I]
     L.conv2d_single_host.argtypes = [P, I, I, P, I, P, P, I]
     L.conv2d_multi_tc.argtypes = [P, I, I, I, I, P, I, I, P, P]
     L.conv2d_release_scratch.argtypes = []
-    for f in ("conv2d_single", "conv2d_single_ex", "conv2d_single_direct", "conv2d_multi",
+    for f in ("conv2d_single", "conv2d_single_ex", "conv2d_single_halo", "conv2d_single_direct", "conv2d_multi",
               "conv2d_multi_ex", "conv2d_single_host", "conv2d_multi_tc", "conv2d_release_scratch",
               "conv2d_version"):
         getattr(L, f).restype = I
@@ -58,6 +60,11 @@ def load(path: str | None = None):
     L.conv2d_strerror.restype = ctypes.c_char_p
     _lib = L
     return L
+
+
+def lib():
+    """The loaded library (hot path: one global lookup instead of load()'s checks)."""
+    return _lib if _lib is not None else load()
 
 
 def strerror(code: int) -> str:
@@ -76,6 +83,10 @@ def conv2d_single(in_ptr, H, W, filt_ptr, K, out_ptr, stream=0) -> int:
 
 def conv2d_single_ex(in_ptr, H, W, filt_ptr, K, out_ptr, stream=0, band_h=0) -> int:
     return load().conv2d_single_ex(in_ptr, H, W, filt_ptr, K, out_ptr, stream, band_h)
+
+
+def conv2d_single_halo(in_ptr, H, W, halo_ptr, halo_rows, filt_ptr, K, out_ptr, stream=0) -> int:
+    return load().conv2d_single_halo(in_ptr, H, W, halo_ptr, halo_rows, filt_ptr, K, out_ptr, stream)
 
 
 def conv2d_single_direct(in_ptr, H, W, filt_ptr, K, out_ptr, stream=0) -> int:

@@ -17,9 +17,33 @@ import torch
 from . import _capi
 
 
-def _stream_handle(stream) -> int:
-    s = stream if stream is not None else torch.cuda.current_stream()
-    return int(s.cuda_stream)
+_raw_stream = torch._C._cuda_getCurrentRawStream  # current stream handle of a device index (no Stream object)
+
+
+def _stream_handle(stream, device_index: int) -> int:
+    if stream is None:
+        return _raw_stream(device_index)
+    return int(stream.cuda_stream)
+
+
+class _on_device:
+    """`with torch.cuda.device(i)` only when i is not already current (the context manager costs
+    several microseconds per call, which is most of a small convolution's host time)."""
+    __slots__ = ("idx", "prev")
+
+    def __init__(self, idx: int):
+        self.idx = idx
+        self.prev = -1
+
+    def __enter__(self):
+        cur = torch.cuda.current_device()
+        if cur != self.idx:
+            self.prev = cur
+            torch.cuda.set_device(self.idx)
+
+    def __exit__(self, *exc):
+        if self.prev >= 0:
+            torch.cuda.set_device(self.prev)
 
 
 def _check_dev(t: torch.Tensor, name: str):
@@ -47,9 +71,40 @@ def conv2d_single(x: torch.Tensor, f: torch.Tensor, out: torch.Tensor | None = N
         _check_dev(out, "out")
         if tuple(out.shape) != (H - K + 1, W - K + 1):
             raise ValueError("out has the wrong shape")
-    with torch.cuda.device(x.device):
-        _capi.check(_capi.conv2d_single_ex(x.data_ptr(), H, W, f.data_ptr(), K, out.data_ptr(),
-                                           _stream_handle(stream), band_h))
+    dev = x.device.index
+    with _on_device(dev):
+        rc = _capi.lib().conv2d_single_ex(x.data_ptr(), H, W, f.data_ptr(), K, out.data_ptr(),
+                                          _stream_handle(stream, dev), band_h)
+    if rc:
+        _capi.check(rc)
+    return out
+
+
+def conv2d_single_halo(x: torch.Tensor, halo: torch.Tensor, f: torch.Tensor, out: torch.Tensor | None = None,
+                       stream=None) -> torch.Tensor:
+    """conv2d_single of the rows of x followed by the rows of halo (same width), without concatenating
+    them: the kernels read the halo rows where they are -- e.g. a peer GPU's band buffer mapped over
+    NVLink (symmetric memory) -- so a row band is one launch. Bitwise equal to
+    conv2d_single(torch.cat([x, halo])). include/conv2d.h: conv2d_single_halo."""
+    _check_dev(x, "x")
+    _check_dev(halo, "halo")
+    _check_dev(f, "f")
+    if x.dim() != 2 or halo.dim() != 2 or halo.shape[1] != x.shape[1] or f.dim() != 2 or f.shape[0] != f.shape[1]:
+        raise ValueError("x must be (H, W), halo (Hh, W) and f (K, K)")
+    H, W = x.shape
+    Hh = halo.shape[0]
+    K = f.shape[0]
+    shape = (max(H + Hh - K + 1, 0), max(W - K + 1, 0))
+    if out is None:
+        out = torch.empty(shape, dtype=torch.float32, device=x.device)
+    else:
+        _check_dev(out, "out")
+        if tuple(out.shape) != shape:
+            raise ValueError("out has the wrong shape")
+    dev = x.device.index
+    with _on_device(dev):
+        _capi.check(_capi.conv2d_single_halo(x.data_ptr(), H, W, halo.data_ptr() if Hh else 0, Hh, f.data_ptr(), K,
+                                             out.data_ptr(), _stream_handle(stream, dev)))
     return out
 
 
@@ -62,9 +117,10 @@ def conv2d_single_direct(x: torch.Tensor, f: torch.Tensor, out: torch.Tensor | N
     K = f.shape[0]
     if out is None:
         out = torch.empty((H - K + 1, W - K + 1), dtype=torch.float32, device=x.device)
-    with torch.cuda.device(x.device):
+    dev = x.device.index
+    with _on_device(dev):
         _capi.check(_capi.conv2d_single_direct(x.data_ptr(), H, W, f.data_ptr(), K, out.data_ptr(),
-                                               _stream_handle(stream)))
+                                               _stream_handle(stream, dev)))
     return out
 
 
@@ -82,9 +138,12 @@ def conv2d_multi(x: torch.Tensor, w: torch.Tensor, out: torch.Tensor | None = No
         _check_dev(out, "out")
         if tuple(out.shape) != (N, F, H - K + 1, W - K + 1):
             raise ValueError("out has the wrong shape")
-    with torch.cuda.device(x.device):
-        _capi.check(_capi.conv2d_multi_ex(x.data_ptr(), N, C, H, W, w.data_ptr(), F, K, out.data_ptr(),
-                                          _stream_handle(stream), band_h))
+    dev = x.device.index
+    with _on_device(dev):
+        rc = _capi.lib().conv2d_multi_ex(x.data_ptr(), N, C, H, W, w.data_ptr(), F, K, out.data_ptr(),
+                                         _stream_handle(stream, dev), band_h)
+    if rc:
+        _capi.check(rc)
     return out
 
 
@@ -98,9 +157,10 @@ def conv2d_multi_tc(x: torch.Tensor, w: torch.Tensor, out: torch.Tensor | None =
     F, _, K, _ = w.shape
     if out is None:
         out = torch.empty((N, F, max(H - K + 1, 0), max(W - K + 1, 0)), dtype=torch.float32, device=x.device)
-    with torch.cuda.device(x.device):
+    dev = x.device.index
+    with _on_device(dev):
         _capi.check(_capi.conv2d_multi_tc(x.data_ptr(), N, C, H, W, w.data_ptr(), F, K, out.data_ptr(),
-                                          _stream_handle(stream)))
+                                          _stream_handle(stream, dev)))
     return out
 
 

@@ -144,9 +144,34 @@ int conv2d_single_ex(const float *in, int H, int W, const float *filt, int K, fl
   DevInfo dev;
   if (current_device_info(&dev)) return CONV2D_ECUDA;
   cudaStream_t s = static_cast<cudaStream_t>(stream);
-#define C2D_CALL_SINGLE(KK) single_entry<KK>(in, H, W, filt, out, s, band_h, dev)
+#define C2D_CALL_SINGLE(KK) single_entry<KK>(in, H, W, filt, out, s, band_h, dev, in, H)
   C2D_K_SWITCH(K, C2D_CALL_SINGLE)
 #undef C2D_CALL_SINGLE
+}
+
+int conv2d_single_halo(const float *in, int H, int W, const float *halo, int halo_rows, const float *filt, int K,
+                       float *out, void *stream) {
+  if (halo_rows < 0) return CONV2D_ESHAPE;
+  if (halo_rows == 0) return conv2d_single_ex(in, H, W, filt, K, out, stream, 0);
+  if (!in || !halo || !filt || !out) return CONV2D_ENULL;
+  if (int e = check_k(K)) return e;
+  if (H < 1 || W < K) return CONV2D_ESHAPE;
+  const long long Ht = static_cast<long long>(H) + halo_rows;
+  if (Ht < K || Ht > 0x7fffffffLL) return CONV2D_ESHAPE;
+  if (!aligned4(in) || !aligned4(halo) || !aligned4(filt) || !aligned4(out)) return CONV2D_EALIGN;
+  const size_t in_b = static_cast<size_t>(H) * W * sizeof(float);
+  const size_t halo_b = static_cast<size_t>(halo_rows) * W * sizeof(float);
+  const size_t out_b = static_cast<size_t>(Ht - K + 1) * (W - K + 1) * sizeof(float);
+  const size_t f_b = static_cast<size_t>(K) * K * sizeof(float);
+  if (overlap(in, in_b, out, out_b) || overlap(halo, halo_b, out, out_b) || overlap(filt, f_b, out, out_b))
+    return CONV2D_EOVERLAP;
+  DevInfo dev;
+  if (current_device_info(&dev)) return CONV2D_ECUDA;
+  cudaStream_t s = static_cast<cudaStream_t>(stream);
+  const int Hi = static_cast<int>(Ht);
+#define C2D_CALL_HALO(KK) single_entry<KK>(in, Hi, W, filt, out, s, 0, dev, halo, H)
+  C2D_K_SWITCH(K, C2D_CALL_HALO)
+#undef C2D_CALL_HALO
 }
 
 int conv2d_single(const float *in, int H, int W, const float *filt, int K, float *out, void *stream) {

@@ -344,6 +344,8 @@ __device__ __forceinline__ void row_step1(float (&acc)[K][U][4], const float (&w
 // ------------------------------------------------------------------------------------------------
 struct SingleArgs {
   const float *in;
+  const float *in2;  // rows >= H1 come from in2 (the halo of a row band, possibly a peer GPU's memory)
+  int H1;            // rows [0, H1) at in, rows [H1, H) at in2 (H1 == H: one segment)
   const float *filt;
   float *out;
   int H, W, Ho, Wo;
@@ -354,7 +356,7 @@ struct SingleArgs {
 };
 
 __device__ __forceinline__ const float *in_row(const SingleArgs &a, int r) {
-  return a.in + static_cast<size_t>(r) * a.W;
+  return r < a.H1 ? a.in + static_cast<size_t>(r) * a.W : a.in2 + static_cast<size_t>(r - a.H1) * a.W;
 }
 __device__ __forceinline__ float *out_row(const SingleArgs &a, int o) {
   return a.out + static_cast<size_t>(o) * a.Wo;

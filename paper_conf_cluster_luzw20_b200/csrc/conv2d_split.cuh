@@ -32,6 +32,8 @@ namespace c2d {
 
 struct SplitArgs {
   const float *in;
+  const float *in2;  // rows >= H1 at in2 (row-band halo), as SingleArgs
+  int H1;
   float *out;
   int H, W, Ho, Wo;
   int band_h;   // output rows per cluster tile
@@ -165,7 +167,9 @@ __device__ __forceinline__ void split_tile(const SplitArgs &a, const FilterSrc<K
   ring.sl = lane;
   constexpr bool clamp = (EDGE == 1);
   RowBuf<K, U> n1;
-  auto in_row_p = [&](int r) { return a.in + static_cast<size_t>(r) * a.W; };
+  auto in_row_p = [&](int r) {
+    return r < a.H1 ? a.in + static_cast<size_t>(r) * a.W : a.in2 + static_cast<size_t>(r - a.H1) * a.W;
+  };
   if constexpr (NST > 1) {
 #pragma unroll
     for (int st = 0; st < NST - 1; ++st) ring.issue(st, in_row_p(min(r0 + st, rlast)), x0, a.W, clamp);

@@ -92,13 +92,15 @@ bool stream_capturing(cudaStream_t s) {
 
 template <int K, int U, int FSRC, int PF = 1, int GUARDS = 0>
 int launch_single_v(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                    const DevInfo &dev, int min_band) {
+                    const DevInfo &dev, int min_band, const float *in2, int H1) {
   constexpr int CTAW = (FSRC == FSRC_CONST) ? 1 : kCtaWarps;
   auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS>;
   static std::atomic<int> occ_cache{0};
   const size_t ring = (PF >= 3) ? CTAW * RowRing<K, U, kWarp, (PF >= 3 ? PF : 2)>::kBytes : 0;
   SingleArgs a;
   a.in = in;
+  a.in2 = in2;
+  a.H1 = H1;
   a.filt = filt;
   a.out = out;
   a.H = H;
@@ -106,7 +108,7 @@ int launch_single_v(const float *in, int H, int W, const float *filt, float *out
   a.Ho = H - K + 1;
   a.Wo = W - K + 1;
   a.n_cb = ceil_div(a.Wo, 128 * U);
-  a.aligned = (aligned16(in) && (W % 4 == 0)) ? 1 : 0;
+  a.aligned = (aligned16(in) && aligned16(in2) && (W % 4 == 0)) ? 1 : 0;
   if (band_h <= 0) {
     // one full wave of warp tiles: bands = resident warps / column blocks
     const long long resident_warps =
@@ -133,7 +135,7 @@ int launch_single_v(const float *in, int H, int W, const float *filt, float *out
 // G times fewer, taller bands.
 template <int K, int G, int U, int PF, int R, int GUARDS, int CL>
 int launch_split_v(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                   const DevInfo &dev, int min_band) {
+                   const DevInfo &dev, int min_band, const float *in2, int H1) {
   static_assert(G >= 1 && G <= 8 && G <= K, "portable cluster of at most K CTAs");
   auto kernel = k_conv2d_split<K, G, U, PF, R, GUARDS, CL>;
   static std::atomic<int> occ_cache{0};
@@ -141,13 +143,15 @@ int launch_split_v(const float *in, int H, int W, const float *filt, float *out,
   const int threads = CL ? kWarp : G * kWarp;
   SplitArgs a;
   a.in = in;
+  a.in2 = in2;
+  a.H1 = H1;
   a.out = out;
   a.H = H;
   a.W = W;
   a.Ho = H - K + 1;
   a.Wo = W - K + 1;
   a.n_cb = ceil_div(a.Wo, 128 * U);
-  a.aligned = (aligned16(in) && (W % 4 == 0)) ? 1 : 0;
+  a.aligned = (aligned16(in) && aligned16(in2) && (W % 4 == 0)) ? 1 : 0;
   static std::atomic<int> smem_set{0};
   if (smem > 48 * 1024 && smem_set.load() == 0) {
     if (smem > static_cast<size_t>(dev.smem_optin)) return CONV2D_ESHAPE;
@@ -207,13 +211,13 @@ int launch_split_v(const float *in, int H, int W, const float *filt, float *out,
 
 template <int K>
 int launch_single(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                  const DevInfo &dev) {
+                  const DevInfo &dev, const float *in2, int H1) {
   const int mb = g_min_band.load(std::memory_order_relaxed);
   const int min_band = mb > 0 ? mb : (K - 1 > 4 ? K - 1 : 4);
   const int v = g_variant.load(std::memory_order_relaxed);
   // CUDA-graph capture cannot use the event-guarded constant slots: shared-memory filter there
   const bool constant_ok = !stream_capturing(stream);
-#define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G>(in, H, W, filt, out, stream, band_h, dev, min_band)
+#define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1)
   switch (v) {
     case 1: return C2D_LS(1, FSRC_SMEM, 1, 0);
     case 2: return C2D_LS(2, FSRC_SMEM, 1, 0);
@@ -228,7 +232,7 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
   }
   // filter-row split (conv2d_split.cuh; variants 10-12)
 #define C2D_SP(GG, UU, PFF, RR, CLL) \
-  launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(in, H, W, filt, out, stream, band_h, dev, 1)
+  launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(in, H, W, filt, out, stream, band_h, dev, 1, in2, H1)
   if (constant_ok && v >= 10 && v <= 12) {
     if constexpr (K >= 3) {
       switch (v) {
@@ -255,7 +259,12 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
   //   K = 10, 11    one chunk + ring + guards;
   //   K >= 12       one chunk, register row fetch, guarded prologue on wide images (tall bands),
   //                 guarded prologue + epilogue on narrow ones.
-  if (!constant_ok) return (K <= 7) ? C2D_LS(2, FSRC_SMEM, 1, 0) : C2D_LS(1, FSRC_SMEM, 1, 0);
+  // Small images with K < 11 are latency-bound (a few microseconds): the per-CTA shared-memory filter
+  // skips the constant-slot staging (a stream-ordered copy plus two event operations, ~3 us of host
+  // and device time per call, tools/host_overhead.py). Same summation order, same bits.
+  const bool small = static_cast<long long>(H) * W <= 512LL * 512;
+  if (!constant_ok || (K < 11 && small && v == 0))
+    return (K <= 7) ? C2D_LS(2, FSRC_SMEM, 1, 0) : C2D_LS(1, FSRC_SMEM, 1, 0);
   if constexpr (K <= 5) {
     if (K <= 3 && W > 1024) return C2D_LS(2, FSRC_CONST, 1, 0);
     return C2D_LS(2, FSRC_CONST, 4, 0);
@@ -437,8 +446,8 @@ namespace c2d {
 
 template <int K>
 int single_entry(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                 const DevInfo &dev) {
-  return launch_single<K>(in, H, W, filt, out, stream, band_h, dev);
+                 const DevInfo &dev, const float *in2, int H1) {
+  return launch_single<K>(in, H, W, filt, out, stream, band_h, dev, in2, H1);
 }
 
 template <int K>

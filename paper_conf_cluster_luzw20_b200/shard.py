@@ -14,6 +14,12 @@ partitions below come from BASELINE.json north_star / configs[3..4]:
                   from 2(K-1) input rows. Outputs are bitwise equal to a one-GPU run (each output's
                   summation order does not depend on where its rows sit; tests pin this).
 
+Fused halo: with the band buffers in symmetric memory (every rank maps its
+neighbours' buffers over NVLink), rank p reads rank p+1's first K-1 rows IN PLACE: one
+conv2d_single_halo launch computes the whole band, the halo rows streaming over NVLink inside the
+kernel's row fetches -- no exchange step, no tail call (`rowband_conv2d_single_p2p`,
+`symmetric_band_buffers`).
+
 `compute` defaults to the CUDA C-ABI call; tests on CPU (gloo) pass the oracle instead -- the
 product path itself has no CPU fallback.
 """
@@ -123,4 +129,46 @@ def rowband_conv2d_single(buf: torch.Tensor, f: torch.Tensor, band: RowBand, out
     # tail: output rows [o1-K+1, o1) from input rows [o1-K+1, o1+K-1): K-1 own + K-1 halo rows
     t0 = max(interior, 0)
     compute(buf[t0:rows + h], f, out[t0:])
+    return out
+
+
+def _default_compute_halo(x: torch.Tensor, halo: torch.Tensor, f: torch.Tensor, out: torch.Tensor) -> None:
+    from .api import conv2d_single_halo
+
+    conv2d_single_halo(x, halo, f, out=out)
+
+
+def symmetric_band_buffers(band: RowBand, device, group=None):
+    """Allocate this rank's band buffer in symmetric memory and map rank+1's first K-1 rows.
+
+    Returns (buf, peer_halo, handle): buf is (band.in_rows, W) local memory every rank can map;
+    peer_halo is a (K-1, W) view of rank+1's buf in this device's address space (None on the last
+    rank); handle is the symmetric-memory handle (handle.barrier() orders a neighbour's writes before
+    our reads). Needs CUDA peer access between the ranks' GPUs (NVLink / NVSwitch)."""
+    import torch.distributed._symmetric_memory as symm_mem
+
+    group = group or dist.group.WORLD
+    buf = symm_mem.empty((band.in_rows, band.W), dtype=torch.float32, device=device)
+    handle = symm_mem.rendezvous(buf, group.group_name)
+    peer = None
+    if not band.is_last and band.halo > 0:
+        peer = handle.get_buffer(band.rank + 1, (band.halo, band.W), torch.float32)
+    return buf, peer, handle
+
+
+def rowband_conv2d_single_p2p(buf: torch.Tensor, peer_halo, f: torch.Tensor, band: RowBand, out: torch.Tensor,
+                              compute_halo=_default_compute_halo, compute=_default_compute) -> torch.Tensor:
+    """Row-band convolution with the halo read in place from the neighbour (one launch per rank).
+
+    buf: (>= band.in_rows, W) this rank's input rows; peer_halo: the first K-1 input rows of rank+1
+    (a peer-memory view from symmetric_band_buffers, or any (K-1, W) tensor holding them); ignored on
+    the last rank. The caller orders the neighbour's writes of those rows before this call (e.g.
+    handle.barrier()); the rows must stay unchanged until the kernel completes.
+    out: (band.out_rows, W-K+1) output rows [o0, o1)."""
+    rows, h = band.out_rows, band.halo
+    assert out.shape[0] == rows
+    if band.is_last or h == 0:
+        compute(buf[:rows + h], f, out)
+    else:
+        compute_halo(buf[:rows], peer_halo, f, out)
     return out

@@ -289,3 +289,34 @@ def test_host_buffer_pipeline(cuda_device, pinned):
             out = pkg.conv2d_single_host(x, f, chunk_rows=chunk)
             torch.cuda.synchronize()
             assert torch.equal(out, ref), (H, W, K, chunk)
+
+
+@pytest.mark.parametrize("K", [1, 3, 7, 12, 15])
+def test_halo_segment_bitwise(cuda_device, K):
+    """conv2d_single_halo (row-band halo read in place): the rows of x followed by
+    the rows of a SEPARATE allocation give the same bits as conv2d_single on the concatenation, for
+    halo_rows 0..K-1 and more, narrow (split kernel) and wide images, aligned and misaligned halos."""
+    f = _filt(K, "rand", seed=K)
+    for (H, W) in [(40, 301), (K + 70, 1030), (200, 2052)]:
+        full = dev_image((H + K + 3, W), "img", seed=K + W)
+        for hr in sorted({0, 1, max(K - 1, 0), K + 3}):
+            x = full[:H].clone()
+            halo_store = torch.empty(((hr + 1) * W + 3,), device=DEV)
+            for off in (0, 1):  # off=1: the halo rows start 4 bytes past a 16-byte boundary
+                halo = halo_store[off:off + hr * W].view(hr, W)
+                halo.copy_(full[H:H + hr])
+                if H + hr < K:
+                    continue
+                ref = pkg.conv2d_single(full[:H + hr].contiguous(), f)
+                got = pkg.conv2d_single_halo(x, halo, f)
+                torch.cuda.synchronize()
+                assert torch.equal(got, ref), (K, H, W, hr, off)
+    x = dev_image((30, 64), "img")
+    halo = dev_image((K, 64), "img", seed=5)
+    y = torch.empty((30 + K - K + 1, 64 - K + 1), device=DEV)
+    assert _capi.conv2d_single_halo(x.data_ptr(), 30, 64, 0, 2, _filt(K).data_ptr(), K, y.data_ptr()) == \
+        _capi.CONV2D_ENULL
+    assert _capi.conv2d_single_halo(x.data_ptr(), 30, 64, halo.data_ptr(), -1, _filt(K).data_ptr(), K,
+                                    y.data_ptr()) == _capi.CONV2D_ESHAPE
+    assert _capi.conv2d_single_halo(x.data_ptr(), 30, 64, halo.data_ptr(), K, _filt(K).data_ptr(), K,
+                                    halo.data_ptr()) == _capi.CONV2D_EOVERLAP

@@ -82,6 +82,49 @@ def test_rowband_halo_exchange_gloo(world, K):
     assert np.array_equal(got, ref)
 
 
+def _oracle_compute_halo(x, halo, f, out):
+    _oracle_compute(torch.cat([x, halo]), f, out)
+
+
+def _worker_rowband_p2p(rank, world, port, H, W, K, tmpdir):
+    """The fused-halo path: each rank reads rank+1's first K-1 rows where they are. On CPU the
+    peer-memory view is stood in for by a separate tensor filled over gloo (symmetric memory needs
+    GPUs); the compute call gets own rows and halo as two separate segments."""
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        band = shard.row_band(H, W, K, world, rank)
+        buf = torch.from_numpy(synth.fill_np(11, synth.TAG_INPUT, (band.in_rows, W), "img", start=band.o0 * W))
+        f = torch.from_numpy(synth.make_filter(11, K, "rand")[0, 0])
+        peer = torch.full((band.halo, W), float("nan"))
+        ops = []
+        if rank > 0 and band.halo:
+            ops.append(dist.P2POp(dist.isend, buf[:band.halo].contiguous(), rank - 1))
+        if not band.is_last and band.halo:
+            ops.append(dist.P2POp(dist.irecv, peer, rank + 1))
+        for r in (dist.batch_isend_irecv(ops) if ops else []):
+            r.wait()
+        out = torch.empty((band.out_rows, W - K + 1))
+        shard.rowband_conv2d_single_p2p(buf, peer, f, band, out, compute_halo=_oracle_compute_halo,
+                                        compute=_oracle_compute)
+        np.save(os.path.join(tmpdir, f"band{rank}.npy"), out.numpy())
+    finally:
+        dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("world,K", [(2, 5), (3, 15), (2, 1)])
+def test_rowband_p2p_halo_gloo(world, K):
+    import oracle
+
+    H, W = 64, 37
+    with tempfile.TemporaryDirectory() as tmp:
+        mp.spawn(_worker_rowband_p2p, args=(world, _free_port(), H, W, K, tmp), nprocs=world, join=True)
+        got = np.concatenate([np.load(os.path.join(tmp, f"band{r}.npy")) for r in range(world)])
+    x = synth.fill_np(11, synth.TAG_INPUT, (H, W), "img")
+    ref, _, _ = oracle.conv2d_single(x, synth.make_filter(11, K, "rand")[0, 0])
+    assert np.array_equal(got, ref)
+
+
 def _worker_batch(rank, world, port, tmpdir):
     import oracle
 
