@@ -45,7 +45,10 @@ def load(path: str | None = None):
     P, I = ctypes.c_void_p, ctypes.c_int
     L.conv2d_single.argtypes = [P, I, I, P, I, P, P]
     L.conv2d_single_ex.argtypes = [P, I, I, P, I, P, P, I]
-    L.conv2d_single_halo.argtypes = [P, I, I, P, I, P, I, P, P]
+    if path is None and "C2D_LIB" in os.environ and not hasattr(L, "conv2d_single_halo"):
+        pass  # an older tuning build (A/B timing only)
+    else:
+        L.conv2d_single_halo.argtypes = [P, I, I, P, I, P, I, P, P]
     L.conv2d_single_direct.argtypes = [P, I, I, P, I, P, P]
     L.conv2d_multi.argtypes = [P, I, I, I, I, P, I, I, P, P]
     L.conv2d_multi_ex.argtypes = [P, I, I, I, I, P, I, I, P, P, I]
@@ -55,7 +58,8 @@ def load(path: str | None = None):
     for f in ("conv2d_single", "conv2d_single_ex", "conv2d_single_halo", "conv2d_single_direct", "conv2d_multi",
               "conv2d_multi_ex", "conv2d_single_host", "conv2d_multi_tc", "conv2d_release_scratch",
               "conv2d_version"):
-        getattr(L, f).restype = I
+        if hasattr(L, f):
+            getattr(L, f).restype = I
     L.conv2d_strerror.argtypes = [I]
     L.conv2d_strerror.restype = ctypes.c_char_p
     _lib = L

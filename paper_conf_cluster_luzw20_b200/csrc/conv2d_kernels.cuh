@@ -355,8 +355,14 @@ struct SingleArgs {
   int aligned;    // in is 16B aligned and W % 4 == 0
 };
 
+// HALO: rows >= H1 come from in2 (conv2d_single_halo); a separate instantiation, so the one-segment
+// kernels keep their row addressing (the per-row select measured -2% at K = 11..15).
+template <bool HALO>
 __device__ __forceinline__ const float *in_row(const SingleArgs &a, int r) {
-  return r < a.H1 ? a.in + static_cast<size_t>(r) * a.W : a.in2 + static_cast<size_t>(r - a.H1) * a.W;
+  if constexpr (HALO)
+    return r < a.H1 ? a.in + static_cast<size_t>(r) * a.W : a.in2 + static_cast<size_t>(r - a.H1) * a.W;
+  else
+    return a.in + static_cast<size_t>(r) * a.W;
 }
 __device__ __forceinline__ float *out_row(const SingleArgs &a, int o) {
   return a.out + static_cast<size_t>(o) * a.Wo;
@@ -378,7 +384,7 @@ __device__ __forceinline__ float *out_row(const SingleArgs &a, int o) {
 // loads, masked scalar stores); 2: misaligned rows (guarded scalar loads, masked stores).
 // PF 1/2: rows r+1 (r+2) in flight in registers; PF >= 3 (power of two, EDGE < 2): a PF-stage cp.async
 // ring in shared memory with PF-1 rows in flight (latency-bound short bands and HBM-bound small K).
-template <int K, int U, int FSRC, int PF, int GUARDS, int EDGE>
+template <int K, int U, int FSRC, int PF, int GUARDS, int EDGE, bool HALO>
 __device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc<K, FSRC> &fs, int x0, int ob,
                                             int oe, int lane, unsigned ring_base) {
   constexpr bool SAFE = (EDGE != 0);
@@ -402,10 +408,10 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc
   RowBuf<K, U> n1, n2;  // register path: rows r+1 (and r+2 when RPF == 2) in flight
   if constexpr (NST > 1) {
 #pragma unroll
-    for (int st = 0; st < NST - 1; ++st) ring.issue(st, in_row(a, min(ob + st, rlast)), x0, a.W, clamp);
+    for (int st = 0; st < NST - 1; ++st) ring.issue(st, in_row<HALO>(a, min(ob + st, rlast)), x0, a.W, clamp);
   } else {
-    load_row<K, U, SAFE>(n1, in_row(a, ob), x0, a.W, lane, a.aligned);
-    if (RPF == 2) load_row<K, U, SAFE>(n2, in_row(a, min(ob + 1, rlast)), x0, a.W, lane, a.aligned);
+    load_row<K, U, SAFE>(n1, in_row<HALO>(a, ob), x0, a.W, lane, a.aligned);
+    if (RPF == 2) load_row<K, U, SAFE>(n2, in_row<HALO>(a, min(ob + 1, rlast)), x0, a.W, lane, a.aligned);
   }
   // returns row r and issues the fetch of row r+depth (index clamped)
   auto next_row = [&](int r) {
@@ -414,14 +420,14 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc
       cp_async_wait<NST - 2>();
       const int k = r - ob;
       ring.read(k & (NST - 1), cur);
-      ring.issue((k + NST - 1) & (NST - 1), in_row(a, min(r + NST - 1, rlast)), x0, a.W, clamp);
+      ring.issue((k + NST - 1) & (NST - 1), in_row<HALO>(a, min(r + NST - 1, rlast)), x0, a.W, clamp);
     } else if constexpr (RPF == 2) {
       cur = n1;
       n1 = n2;
-      load_row<K, U, SAFE>(n2, in_row(a, min(r + 2, rlast)), x0, a.W, lane, a.aligned);
+      load_row<K, U, SAFE>(n2, in_row<HALO>(a, min(r + 2, rlast)), x0, a.W, lane, a.aligned);
     } else {
       cur = n1;
-      load_row<K, U, SAFE>(n1, in_row(a, min(r + 1, rlast)), x0, a.W, lane, a.aligned);
+      load_row<K, U, SAFE>(n1, in_row<HALO>(a, min(r + 1, rlast)), x0, a.W, lane, a.aligned);
     }
     return cur;
   };
@@ -462,7 +468,7 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc
 // CTAW: warps per CTA. With CTAW == 1 every branch depends only on blockIdx and kernel parameters,
 // so the compiler can prove warp-uniform control flow and keep the constant-bank filter in uniform
 // registers (LDCU + FFMA with UR operands) instead of per-lane loads.
-template <int K, int U, int FSRC, int CTAW, int PF = 1, int GUARDS = 0>
+template <int K, int U, int FSRC, int CTAW, int PF = 1, int GUARDS = 0, bool HALO = false>
 __global__ void __launch_bounds__(CTAW *kWarp) k_conv2d_single(const SingleArgs a) {
   constexpr int KP = KCfg<K>::KP;
   __shared__ __align__(16) float sf[(FSRC == FSRC_SMEM) ? K * KP : 4];
@@ -492,11 +498,11 @@ __global__ void __launch_bounds__(CTAW *kWarp) k_conv2d_single(const SingleArgs 
   // fast tiles: 16B-aligned rows, every column of the tile and its extra halo quad in range
   const bool inside = x0 + 128 * U + 4 * KCfg<K>::NE <= a.W;  // warp-uniform
   if (a.aligned && inside)
-    single_tile<K, U, FSRC, PF, GUARDS, 0>(a, fs, x0, ob, oe, lane, ring_base);
+    single_tile<K, U, FSRC, PF, GUARDS, 0, HALO>(a, fs, x0, ob, oe, lane, ring_base);
   else if (a.aligned)
-    single_tile<K, U, FSRC, PF, GUARDS, 1>(a, fs, x0, ob, oe, lane, ring_base);
+    single_tile<K, U, FSRC, PF, GUARDS, 1, HALO>(a, fs, x0, ob, oe, lane, ring_base);
   else
-    single_tile<K, U, FSRC, PF, GUARDS, 2>(a, fs, x0, ob, oe, lane, ring_base);
+    single_tile<K, U, FSRC, PF, GUARDS, 2, HALO>(a, fs, x0, ob, oe, lane, ring_base);
 }
 
 // ------------------------------------------------------------------------------------------------

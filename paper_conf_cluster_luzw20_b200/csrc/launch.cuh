@@ -90,11 +90,11 @@ bool stream_capturing(cudaStream_t s) {
   return cudaStreamIsCapturing(s, &st) == cudaSuccess && st != cudaStreamCaptureStatusNone;
 }
 
-template <int K, int U, int FSRC, int PF = 1, int GUARDS = 0>
+template <int K, int U, int FSRC, int PF = 1, int GUARDS = 0, bool HALO = false>
 int launch_single_v(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
                     const DevInfo &dev, int min_band, const float *in2, int H1) {
   constexpr int CTAW = (FSRC == FSRC_CONST) ? 1 : kCtaWarps;
-  auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS>;
+  auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS, HALO>;
   static std::atomic<int> occ_cache{0};
   const size_t ring = (PF >= 3) ? CTAW * RowRing<K, U, kWarp, (PF >= 3 ? PF : 2)>::kBytes : 0;
   SingleArgs a;
@@ -217,6 +217,17 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
   const int v = g_variant.load(std::memory_order_relaxed);
   // CUDA-graph capture cannot use the event-guarded constant slots: shared-memory filter there
   const bool constant_ok = !stream_capturing(stream);
+  if (H1 < H) {
+    // conv2d_single_halo: the halo instantiations (same sums as every one-tile variant: same bits),
+    // or the split kernel where the default takes it (it addresses both segments natively)
+    if constexpr (K >= 11) {
+      if (constant_ok && W <= 1024) return launch_split_v<K, 2, 1, 4, 4, 1, 1>(in, H, W, filt, out, stream, band_h,
+                                                                                 dev, 1, in2, H1);
+    }
+    if (!constant_ok)
+      return launch_single_v<K, 1, FSRC_SMEM, 1, 0, true>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1);
+    return launch_single_v<K, 1, FSRC_CONST, 4, 2, true>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1);
+  }
 #define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1)
   switch (v) {
     case 1: return C2D_LS(1, FSRC_SMEM, 1, 0);
