@@ -105,6 +105,30 @@ int conv2d_single_halo(const float *in, int H, int W, const float *halo, int hal
                        int K, float *out, void *stream);
 
 /*
+ * Boundary and semantic variants of conv2d_single (the image-library semantics the
+ * paper compares against). `mode` is a bitwise OR of
+ *   CONV2D_PAD_ZERO      'same' output size H x W, input padded with zeros,
+ *   CONV2D_PAD_REPLICATE 'same' output size H x W, input padded by repeating its edge elements,
+ *                        (at most one PAD flag; padding: top/left (K-1)/2, bottom/right the rest --
+ *                        torch.nn.functional.conv2d(padding='same') placement, also for even K),
+ *   CONV2D_FLIP          true convolution: the filter is rotated by 180 degrees (NPP / ArrayFire /
+ *                        scipy.signal.convolve2d orientation) instead of cross-correlation.
+ * mode == 0 is conv2d_single. Without a PAD flag the output is (H-K+1) x (W-K+1) and H, W >= K is
+ * required; with one, H, W >= 1. Same layouts, ownership, stream semantics and tolerance as
+ * conv2d_single; the result is bitwise equal to conv2d_single on the padded image with the rotated
+ * filter (the padding and the rotation are data movement done on the device into the library's
+ * stream-ordered scratch pool; the convolution is the same per-K kernels).
+ * Errors as conv2d_single, plus CONV2D_ESHAPE for an invalid mode and CONV2D_EALLOC when the scratch
+ * pool cannot provide the padded image ((H+K-1) x (W+K-1) floats, row pitch rounded to 16 bytes).
+ */
+#define CONV2D_PAD_ZERO 1
+#define CONV2D_PAD_REPLICATE 2
+#define CONV2D_PAD_MASK 3
+#define CONV2D_FLIP 4
+int conv2d_single_pad(const float *in, int H, int W, const float *filt, int K, int mode, float *out,
+                      void *stream);
+
+/*
  * Baseline "direct convolution" of PAPER.md Fig. 1a: one thread per
  * output element, each thread loads its K*K inputs itself (no column or row reuse). Same arguments,
  * result and error codes as conv2d_single. Kept as the control for the memory-transaction evidence

@@ -139,6 +139,42 @@ def conv2d_multi_points(inp, filt, ns, fs, ys, xs):
     return out, bound
 
 
+def extend_image(image, K, padding):
+    """The image extended by K-1 rows and columns for 'same' output (reading R20):
+    E[r][c] = image[r - pt][c - pl] with pt = pl = (K-1)//2 (bottom / right get K-1-(K-1)//2, the
+    torch padding='same' placement); outside the image E is 0 ("same_zero") or the nearest edge
+    element ("same_replicate"). Written as an index map, element by element."""
+    image = _f32(image)
+    H, W = image.shape
+    pt = (K - 1) // 2
+    rows = np.arange(H + K - 1) - pt
+    cols = np.arange(W + K - 1) - pt
+    if padding == "same_replicate":
+        return image[np.clip(rows, 0, H - 1)][:, np.clip(cols, 0, W - 1)]
+    assert padding == "same_zero"
+    E = np.zeros((H + K - 1, W + K - 1), np.float32)
+    ri = (rows >= 0) & (rows < H)
+    ci = (cols >= 0) & (cols < W)
+    E[np.ix_(ri, ci)] = image
+    return E
+
+
+def conv2d_single_pad(image, filt, padding="valid", flip=False):
+    """Boundary / semantic variants (include/conv2d.h conv2d_single_pad):
+
+        out[y][x] = fl32( sum_i sum_j E[y+i][x+j] * g[i][j] )
+
+    with E the image itself ("valid") or extend_image(...) ("same_zero", "same_replicate"), and
+    g = filt (cross-correlation, the paper's orientation, R1) or g[i][j] = filt[K-1-i][K-1-j] (true
+    convolution, flip=True: the NPP / ArrayFire orientation). The sum is the plain
+    definition of conv2d_single above. Returns (out, bound, None)."""
+    filt = _f32(filt)
+    K = filt.shape[0]
+    g = filt[::-1, ::-1] if flip else filt
+    E = _f32(image) if padding == "valid" else extend_image(image, K, padding)
+    return conv2d_single(E, g)
+
+
 def within_tolerance(gpu, ref, bound, rel=1e-5):
     """The BASELINE.json north_star acceptance test |gpu - ref| <= rel * sum|x||w|, elementwise.
 

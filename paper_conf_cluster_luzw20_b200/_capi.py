@@ -10,6 +10,7 @@ LIB_PATH = os.path.join(_PKG, "libconv2d.so")
 
 # every symbol include/conv2d.h declares
 EXPORTS = ("conv2d_single", "conv2d_multi", "conv2d_single_ex", "conv2d_multi_ex", "conv2d_single_halo",
+           "conv2d_single_pad",
            "conv2d_single_direct",
            "conv2d_single_host", "conv2d_multi_tc", "conv2d_release_scratch", "conv2d_strerror", "conv2d_version")
 
@@ -22,6 +23,9 @@ CONV2D_ECUDA = -5
 CONV2D_EALIGN = -6
 CONV2D_EALLOC = -7
 CONV2D_MAX_K = 15
+CONV2D_PAD_ZERO = 1
+CONV2D_PAD_REPLICATE = 2
+CONV2D_FLIP = 4
 
 _lib = None
 
@@ -49,13 +53,15 @@ def load(path: str | None = None):
         pass  # an older tuning build (A/B timing only)
     else:
         L.conv2d_single_halo.argtypes = [P, I, I, P, I, P, I, P, P]
+    if hasattr(L, "conv2d_single_pad"):
+        L.conv2d_single_pad.argtypes = [P, I, I, P, I, I, P, P]
     L.conv2d_single_direct.argtypes = [P, I, I, P, I, P, P]
     L.conv2d_multi.argtypes = [P, I, I, I, I, P, I, I, P, P]
     L.conv2d_multi_ex.argtypes = [P, I, I, I, I, P, I, I, P, P, I]
     L.conv2d_single_host.argtypes = [P, I, I, P, I, P, P, I]
     L.conv2d_multi_tc.argtypes = [P, I, I, I, I, P, I, I, P, P]
     L.conv2d_release_scratch.argtypes = []
-    for f in ("conv2d_single", "conv2d_single_ex", "conv2d_single_halo", "conv2d_single_direct", "conv2d_multi",
+    for f in ("conv2d_single", "conv2d_single_ex", "conv2d_single_halo", "conv2d_single_pad", "conv2d_single_direct", "conv2d_multi",
               "conv2d_multi_ex", "conv2d_single_host", "conv2d_multi_tc", "conv2d_release_scratch",
               "conv2d_version"):
         if hasattr(L, f):
@@ -87,6 +93,10 @@ def conv2d_single(in_ptr, H, W, filt_ptr, K, out_ptr, stream=0) -> int:
 
 def conv2d_single_ex(in_ptr, H, W, filt_ptr, K, out_ptr, stream=0, band_h=0) -> int:
     return load().conv2d_single_ex(in_ptr, H, W, filt_ptr, K, out_ptr, stream, band_h)
+
+
+def conv2d_single_pad(in_ptr, H, W, filt_ptr, K, mode, out_ptr, stream=0) -> int:
+    return load().conv2d_single_pad(in_ptr, H, W, filt_ptr, K, mode, out_ptr, stream)
 
 
 def conv2d_single_halo(in_ptr, H, W, halo_ptr, halo_rows, filt_ptr, K, out_ptr, stream=0) -> int:

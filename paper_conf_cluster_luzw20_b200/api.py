@@ -108,6 +108,37 @@ def conv2d_single_halo(x: torch.Tensor, halo: torch.Tensor, f: torch.Tensor, out
     return out
 
 
+_PAD_MODES = {"valid": 0, "same": _capi.CONV2D_PAD_ZERO, "same_zero": _capi.CONV2D_PAD_ZERO,
+              "same_replicate": _capi.CONV2D_PAD_REPLICATE}
+
+
+def conv2d_single_pad(x: torch.Tensor, f: torch.Tensor, padding: str = "same", flip: bool = False,
+                      out: torch.Tensor | None = None, stream=None) -> torch.Tensor:
+    """Boundary / semantic variants (include/conv2d.h conv2d_single_pad): padding "valid", "same" (=
+    "same_zero") or "same_replicate"; flip=True for true convolution (rotated filter)."""
+    _check_dev(x, "x")
+    _check_dev(f, "f")
+    if x.dim() != 2 or f.dim() != 2 or f.shape[0] != f.shape[1]:
+        raise ValueError("x must be (H, W) and f (K, K)")
+    if padding not in _PAD_MODES:
+        raise ValueError(f"padding must be one of {sorted(_PAD_MODES)}")
+    mode = _PAD_MODES[padding] | (_capi.CONV2D_FLIP if flip else 0)
+    H, W = x.shape
+    K = f.shape[0]
+    shape = (H, W) if mode & 3 else (max(H - K + 1, 0), max(W - K + 1, 0))
+    if out is None:
+        out = torch.empty(shape, dtype=torch.float32, device=x.device)
+    else:
+        _check_dev(out, "out")
+        if tuple(out.shape) != shape:
+            raise ValueError("out has the wrong shape")
+    dev = x.device.index
+    with _on_device(dev):
+        _capi.check(_capi.conv2d_single_pad(x.data_ptr(), H, W, f.data_ptr(), K, mode, out.data_ptr(),
+                                            _stream_handle(stream, dev)))
+    return out
+
+
 def conv2d_single_direct(x: torch.Tensor, f: torch.Tensor, out: torch.Tensor | None = None,
                          stream=None) -> torch.Tensor:
     """PAPER.md Fig. 1a baseline kernel (no column/row reuse); evidence control only."""

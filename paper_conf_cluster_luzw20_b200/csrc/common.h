@@ -30,7 +30,8 @@ cudaError_t scratch_trim();
 // per-K entry points, explicitly instantiated one K per translation unit (csrc/inst_kNN.cu)
 template <int K>
 int single_entry(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                 const DevInfo &dev, const float *in2, int H1);  // rows >= H1 at in2 (H1 == H: one segment)
+                 const DevInfo &dev, const float *in2, int H1,
+                 long long P);  // rows >= H1 at in2 (H1 == H: one segment); input row pitch P floats
 template <int K>
 int multi_entry(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
                 cudaStream_t stream, int band_h, const DevInfo &dev);

@@ -346,6 +346,8 @@ struct SingleArgs {
   const float *in;
   const float *in2;  // rows >= H1 come from in2 (the halo of a row band, possibly a peer GPU's memory)
   int H1;            // rows [0, H1) at in, rows [H1, H) at in2 (H1 == H: one segment)
+  int P;             // input row pitch in floats (>= W; == W for the C-ABI calls, padded buffers: % 4 == 0)
+  int Wc;            // row-fetch bound: W, or P for a padded buffer (clamped quads stay in the pitch)
   const float *filt;
   float *out;
   int H, W, Ho, Wo;
@@ -360,9 +362,9 @@ struct SingleArgs {
 template <bool HALO>
 __device__ __forceinline__ const float *in_row(const SingleArgs &a, int r) {
   if constexpr (HALO)
-    return r < a.H1 ? a.in + static_cast<size_t>(r) * a.W : a.in2 + static_cast<size_t>(r - a.H1) * a.W;
+    return r < a.H1 ? a.in + static_cast<size_t>(r) * a.P : a.in2 + static_cast<size_t>(r - a.H1) * a.P;
   else
-    return a.in + static_cast<size_t>(r) * a.W;
+    return a.in + static_cast<size_t>(r) * a.P;
 }
 __device__ __forceinline__ float *out_row(const SingleArgs &a, int o) {
   return a.out + static_cast<size_t>(o) * a.Wo;
@@ -408,10 +410,10 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc
   RowBuf<K, U> n1, n2;  // register path: rows r+1 (and r+2 when RPF == 2) in flight
   if constexpr (NST > 1) {
 #pragma unroll
-    for (int st = 0; st < NST - 1; ++st) ring.issue(st, in_row<HALO>(a, min(ob + st, rlast)), x0, a.W, clamp);
+    for (int st = 0; st < NST - 1; ++st) ring.issue(st, in_row<HALO>(a, min(ob + st, rlast)), x0, a.Wc, clamp);
   } else {
-    load_row<K, U, SAFE>(n1, in_row<HALO>(a, ob), x0, a.W, lane, a.aligned);
-    if (RPF == 2) load_row<K, U, SAFE>(n2, in_row<HALO>(a, min(ob + 1, rlast)), x0, a.W, lane, a.aligned);
+    load_row<K, U, SAFE>(n1, in_row<HALO>(a, ob), x0, a.Wc, lane, a.aligned);
+    if (RPF == 2) load_row<K, U, SAFE>(n2, in_row<HALO>(a, min(ob + 1, rlast)), x0, a.Wc, lane, a.aligned);
   }
   // returns row r and issues the fetch of row r+depth (index clamped)
   auto next_row = [&](int r) {
@@ -420,14 +422,14 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc
       cp_async_wait<NST - 2>();
       const int k = r - ob;
       ring.read(k & (NST - 1), cur);
-      ring.issue((k + NST - 1) & (NST - 1), in_row<HALO>(a, min(r + NST - 1, rlast)), x0, a.W, clamp);
+      ring.issue((k + NST - 1) & (NST - 1), in_row<HALO>(a, min(r + NST - 1, rlast)), x0, a.Wc, clamp);
     } else if constexpr (RPF == 2) {
       cur = n1;
       n1 = n2;
-      load_row<K, U, SAFE>(n2, in_row<HALO>(a, min(r + 2, rlast)), x0, a.W, lane, a.aligned);
+      load_row<K, U, SAFE>(n2, in_row<HALO>(a, min(r + 2, rlast)), x0, a.Wc, lane, a.aligned);
     } else {
       cur = n1;
-      load_row<K, U, SAFE>(n1, in_row<HALO>(a, min(r + 1, rlast)), x0, a.W, lane, a.aligned);
+      load_row<K, U, SAFE>(n1, in_row<HALO>(a, min(r + 1, rlast)), x0, a.Wc, lane, a.aligned);
     }
     return cur;
   };

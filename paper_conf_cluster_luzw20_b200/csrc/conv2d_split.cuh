@@ -34,6 +34,8 @@ struct SplitArgs {
   const float *in;
   const float *in2;  // rows >= H1 at in2 (row-band halo), as SingleArgs
   int H1;
+  int P;        // input row pitch in floats, as SingleArgs
+  int Wc;       // row-fetch bound, as SingleArgs
   float *out;
   int H, W, Ho, Wo;
   int band_h;   // output rows per cluster tile
@@ -168,13 +170,13 @@ __device__ __forceinline__ void split_tile(const SplitArgs &a, const FilterSrc<K
   constexpr bool clamp = (EDGE == 1);
   RowBuf<K, U> n1;
   auto in_row_p = [&](int r) {
-    return r < a.H1 ? a.in + static_cast<size_t>(r) * a.W : a.in2 + static_cast<size_t>(r - a.H1) * a.W;
+    return r < a.H1 ? a.in + static_cast<size_t>(r) * a.P : a.in2 + static_cast<size_t>(r - a.H1) * a.P;
   };
   if constexpr (NST > 1) {
 #pragma unroll
-    for (int st = 0; st < NST - 1; ++st) ring.issue(st, in_row_p(min(r0 + st, rlast)), x0, a.W, clamp);
+    for (int st = 0; st < NST - 1; ++st) ring.issue(st, in_row_p(min(r0 + st, rlast)), x0, a.Wc, clamp);
   } else {
-    load_row<K, U, SAFE>(n1, in_row_p(r0), x0, a.W, lane, a.aligned);
+    load_row<K, U, SAFE>(n1, in_row_p(r0), x0, a.Wc, lane, a.aligned);
   }
   int r = r0;
   auto next_row = [&]() {
@@ -183,10 +185,10 @@ __device__ __forceinline__ void split_tile(const SplitArgs &a, const FilterSrc<K
       cp_async_wait<NST - 2>();
       const int k = r - r0;
       ring.read(k & (NST - 1), cur);
-      ring.issue((k + NST - 1) & (NST - 1), in_row_p(min(r + NST - 1, rlast)), x0, a.W, clamp);
+      ring.issue((k + NST - 1) & (NST - 1), in_row_p(min(r + NST - 1, rlast)), x0, a.Wc, clamp);
     } else {
       cur = n1;
-      load_row<K, U, SAFE>(n1, in_row_p(min(r + 1, rlast)), x0, a.W, lane, a.aligned);
+      load_row<K, U, SAFE>(n1, in_row_p(min(r + 1, rlast)), x0, a.Wc, lane, a.aligned);
     }
     return cur;
   };

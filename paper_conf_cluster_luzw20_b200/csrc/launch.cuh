@@ -92,7 +92,7 @@ bool stream_capturing(cudaStream_t s) {
 
 template <int K, int U, int FSRC, int PF = 1, int GUARDS = 0, bool HALO = false>
 int launch_single_v(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                    const DevInfo &dev, int min_band, const float *in2, int H1) {
+                    const DevInfo &dev, int min_band, const float *in2, int H1, long long P) {
   constexpr int CTAW = (FSRC == FSRC_CONST) ? 1 : kCtaWarps;
   auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS, HALO>;
   static std::atomic<int> occ_cache{0};
@@ -101,6 +101,8 @@ int launch_single_v(const float *in, int H, int W, const float *filt, float *out
   a.in = in;
   a.in2 = in2;
   a.H1 = H1;
+  a.P = static_cast<int>(P);
+  a.Wc = static_cast<int>(P);
   a.filt = filt;
   a.out = out;
   a.H = H;
@@ -108,7 +110,7 @@ int launch_single_v(const float *in, int H, int W, const float *filt, float *out
   a.Ho = H - K + 1;
   a.Wo = W - K + 1;
   a.n_cb = ceil_div(a.Wo, 128 * U);
-  a.aligned = (aligned16(in) && aligned16(in2) && (W % 4 == 0)) ? 1 : 0;
+  a.aligned = (aligned16(in) && aligned16(in2) && (P % 4 == 0)) ? 1 : 0;
   if (band_h <= 0) {
     // one full wave of warp tiles: bands = resident warps / column blocks
     const long long resident_warps =
@@ -135,7 +137,7 @@ int launch_single_v(const float *in, int H, int W, const float *filt, float *out
 // G times fewer, taller bands.
 template <int K, int G, int U, int PF, int R, int GUARDS, int CL>
 int launch_split_v(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                   const DevInfo &dev, int min_band, const float *in2, int H1) {
+                   const DevInfo &dev, int min_band, const float *in2, int H1, long long P) {
   static_assert(G >= 1 && G <= 8 && G <= K, "portable cluster of at most K CTAs");
   auto kernel = k_conv2d_split<K, G, U, PF, R, GUARDS, CL>;
   static std::atomic<int> occ_cache{0};
@@ -145,13 +147,15 @@ int launch_split_v(const float *in, int H, int W, const float *filt, float *out,
   a.in = in;
   a.in2 = in2;
   a.H1 = H1;
+  a.P = static_cast<int>(P);
+  a.Wc = static_cast<int>(P);
   a.out = out;
   a.H = H;
   a.W = W;
   a.Ho = H - K + 1;
   a.Wo = W - K + 1;
   a.n_cb = ceil_div(a.Wo, 128 * U);
-  a.aligned = (aligned16(in) && aligned16(in2) && (W % 4 == 0)) ? 1 : 0;
+  a.aligned = (aligned16(in) && aligned16(in2) && (P % 4 == 0)) ? 1 : 0;
   static std::atomic<int> smem_set{0};
   if (smem > 48 * 1024 && smem_set.load() == 0) {
     if (smem > static_cast<size_t>(dev.smem_optin)) return CONV2D_ESHAPE;
@@ -211,7 +215,7 @@ int launch_split_v(const float *in, int H, int W, const float *filt, float *out,
 
 template <int K>
 int launch_single(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                  const DevInfo &dev, const float *in2, int H1) {
+                  const DevInfo &dev, const float *in2, int H1, long long P) {
   const int mb = g_min_band.load(std::memory_order_relaxed);
   const int min_band = mb > 0 ? mb : (K - 1 > 4 ? K - 1 : 4);
   const int v = g_variant.load(std::memory_order_relaxed);
@@ -222,13 +226,13 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
     // or the split kernel where the default takes it (it addresses both segments natively)
     if constexpr (K >= 11) {
       if (constant_ok && W <= 1024) return launch_split_v<K, 2, 1, 4, 4, 1, 1>(in, H, W, filt, out, stream, band_h,
-                                                                                 dev, 1, in2, H1);
+                                                                                 dev, 1, in2, H1, P);
     }
     if (!constant_ok)
-      return launch_single_v<K, 1, FSRC_SMEM, 1, 0, true>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1);
-    return launch_single_v<K, 1, FSRC_CONST, 4, 2, true>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1);
+      return launch_single_v<K, 1, FSRC_SMEM, 1, 0, true>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1, P);
+    return launch_single_v<K, 1, FSRC_CONST, 4, 2, true>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1, P);
   }
-#define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1)
+#define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1, P)
   switch (v) {
     case 1: return C2D_LS(1, FSRC_SMEM, 1, 0);
     case 2: return C2D_LS(2, FSRC_SMEM, 1, 0);
@@ -243,7 +247,7 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
   }
   // filter-row split (conv2d_split.cuh; variants 10-12)
 #define C2D_SP(GG, UU, PFF, RR, CLL) \
-  launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(in, H, W, filt, out, stream, band_h, dev, 1, in2, H1)
+  launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(in, H, W, filt, out, stream, band_h, dev, 1, in2, H1, P)
   if (constant_ok && v >= 10 && v <= 12) {
     if constexpr (K >= 3) {
       switch (v) {
@@ -457,8 +461,8 @@ namespace c2d {
 
 template <int K>
 int single_entry(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                 const DevInfo &dev, const float *in2, int H1) {
-  return launch_single<K>(in, H, W, filt, out, stream, band_h, dev, in2, H1);
+                 const DevInfo &dev, const float *in2, int H1, long long P) {
+  return launch_single<K>(in, H, W, filt, out, stream, band_h, dev, in2, H1, P);
 }
 
 template <int K>

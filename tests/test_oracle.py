@@ -218,3 +218,99 @@ def test_within_tolerance_helper():
     assert oracle.within_tolerance(ref + [1e-6, 0, 0, 0], ref, bound).tolist() == [True, True, True, True]
     assert not oracle.within_tolerance(ref + [2e-5, 0, 0, 0], ref, bound)[0]
     assert not oracle.within_tolerance(ref + [0, 0, 0, 1e-30], ref, bound)[3]
+
+
+
+# ---------------------------------------------------------------------------------------------
+# N4 boundary / semantic variants (oracle.conv2d_single_pad)
+# ---------------------------------------------------------------------------------------------
+@pytest.mark.parametrize("K", [1, 2, 3, 4, 5, 8, 15])
+def test_same_zero_matches_torch_padding_same(K):
+    """'same' zero padding (both odd and even K) == torch.nn.functional.conv2d(padding='same') in f64."""
+    import torch
+
+    rng = np.random.default_rng(K)
+    for (H, W) in [(K + 5, K + 9), (3, 4), (1, 1), (17, 2)]:
+        x = rng.standard_normal((H, W)).astype(np.float32)
+        f = rng.standard_normal((K, K)).astype(np.float32)
+        y, bound, _ = oracle.conv2d_single_pad(x, f, "same_zero")
+        ref = torch.nn.functional.conv2d(torch.from_numpy(x).double()[None, None], torch.from_numpy(f).double()[None, None],
+                                         padding="same")[0, 0].numpy()
+        assert y.shape == (H, W)
+        assert np.allclose(y, ref, rtol=0, atol=1e-6 * (1 + np.abs(ref).max()))
+
+
+@pytest.mark.parametrize("K", [2, 3, 6, 7])
+def test_same_replicate_matches_torch_replicate_pad(K):
+    import torch
+
+    rng = np.random.default_rng(K + 100)
+    x = rng.standard_normal((K + 7, K + 3)).astype(np.float32)
+    f = rng.standard_normal((K, K)).astype(np.float32)
+    y, _, _ = oracle.conv2d_single_pad(x, f, "same_replicate")
+    pt = (K - 1) // 2
+    xp = torch.nn.functional.pad(torch.from_numpy(x).double()[None, None], (pt, K - 1 - pt, pt, K - 1 - pt),
+                                 mode="replicate")
+    ref = torch.nn.functional.conv2d(xp, torch.from_numpy(f).double()[None, None])[0, 0].numpy()
+    assert np.allclose(y, ref, rtol=0, atol=1e-6 * (1 + np.abs(ref).max()))
+
+
+@pytest.mark.parametrize("K", [1, 3, 4, 9])
+def test_flip_matches_scipy_convolve2d(K):
+    """True convolution == scipy.signal.convolve2d (valid), the textbook flipped-kernel definition."""
+    from scipy.signal import convolve2d
+
+    rng = np.random.default_rng(K + 7)
+    x = rng.standard_normal((K + 6, K + 11)).astype(np.float32)
+    f = rng.standard_normal((K, K)).astype(np.float32)
+    y, _, _ = oracle.conv2d_single_pad(x, f, "valid", flip=True)
+    ref = convolve2d(x.astype(np.float64), f.astype(np.float64), mode="valid")
+    assert np.allclose(y, ref, rtol=0, atol=1e-6 * (1 + np.abs(ref).max()))
+
+
+@pytest.mark.parametrize("K", [1, 3, 5, 15])
+def test_same_zero_centered_delta_is_identity(K):
+    """odd K, 'same' zero padding, delta at the centre: every output equals its input (bitwise)."""
+    x = synth.fill_np(5, synth.TAG_INPUT, (K + 4, 2 * K + 3), "sym")
+    f = np.zeros((K, K), np.float32)
+    f[K // 2, K // 2] = 1.0
+    y, _, _ = oracle.conv2d_single_pad(x, f, "same_zero")
+    assert np.array_equal(y, x)
+
+
+@pytest.mark.parametrize("K", [2, 5, 8])
+def test_same_zero_box_filter_counts_window_cells(K):
+    """ones image, box filter, zero padding: out[y][x] = (#rows of the window inside the image) *
+    (#columns inside) -- a closed form of the padding placement (top/left (K-1)//2)."""
+    H, W = K + 3, 2 * K + 1
+    y, _, _ = oracle.conv2d_single_pad(np.ones((H, W), np.float32), np.ones((K, K), np.float32), "same_zero")
+    pt = (K - 1) // 2
+
+    def inside(n, L):
+        return np.array([sum(1 for i in range(K) if 0 <= v + i - pt < L) for v in range(n)], np.float64)
+
+    assert np.array_equal(y, np.outer(inside(H, H), inside(W, W)).astype(np.float32))
+
+
+@pytest.mark.parametrize("K", [3, 4, 7])
+def test_same_replicate_constant_image(K):
+    """replicate padding of a constant image is the constant everywhere: out = c * sum(w), exactly
+    (small integers)."""
+    f = np.arange(K * K, dtype=np.float32).reshape(K, K) - 5
+    y, _, _ = oracle.conv2d_single_pad(np.full((K + 2, K + 5), 3.0, np.float32), f, "same_replicate")
+    assert np.array_equal(y, np.full(y.shape, 3.0 * f.sum(), np.float32))
+
+
+@pytest.mark.parametrize("K", [2, 3, 6])
+def test_flip_impulse_gives_filter_upright(K):
+    """true convolution of an impulse at (r0, c0) is the filter in its own orientation at
+    [r0-K+1, r0] x [c0-K+1, c0] (cross-correlation gives it rotated: test_impulse_input_gives_filter)."""
+    H, W = 3 * K, 3 * K + 1
+    r0, c0 = K + 1, K + 2
+    x = np.zeros((H, W), np.float32)
+    x[r0, c0] = 1.0
+    f = synth.make_filter(3, K, "rand")[0, 0]
+    y, _, _ = oracle.conv2d_single_pad(x, f, "valid", flip=True)
+    exp = np.zeros_like(y)
+    exp[r0 - K + 1:r0 + 1, c0 - K + 1:c0 + 1] = f
+    assert np.array_equal(y, exp)
