@@ -384,14 +384,40 @@ int launch_multi2_v(const float *in, int N, int C, int H, int W, const float *fi
   a.n_fb = ceil_div(F, FB);
   a.n_groups = ceil_div(N, SEGS);
   a.aligned = (aligned16(in) && (W % 4 == 0)) ? 1 : 0;
-  if (band_h <= 0) {
-    // one full wave of resident warps
+  if (band_h <= 0 && K >= 5) {
+    // one full wave of resident warps (tools/multi_band_sweep.py: for K >= 5 the K-1 prologue rows
+    // of extra bands cost more than the wave quantisation they remove -- Table I CONV3/CONV5, configs[3])
     const long long resident_warps =
         static_cast<long long>(cta_occupancy(kernel, smem, occ_cache)) * kCtaWarps * dev.num_sms;
     const long long groups = static_cast<long long>(a.n_groups) * a.n_fb * a.n_cb;
     long long bands = resident_warps / groups;
     if (bands < 1) bands = 1;
     band_h = ceil_div(a.Ho, bands);
+  } else if (band_h <= 0) {
+    // K <= 4: band count by a wave-quantisation cost model: a tile of h output rows streams h + K - 1
+    // input rows, and the grid runs in ceil(CTAs / resident CTAs) waves, so pick the band count b
+    // that minimises waves(b) * (ceil(Ho / b) + K - 1). (One band per tile whenever the (image,
+    // F-block, column-block) groups alone exceed a wave left e.g. Table I CONV11 at 1.15 waves -- 2
+    // waves, the second 15% full: 946 -> 570 us; CONV8/9 2x.)
+    const long long resident_ctas = static_cast<long long>(cta_occupancy(kernel, smem, occ_cache)) * dev.num_sms;
+    const long long groups = static_cast<long long>(a.n_groups) * a.n_fb;
+    long long best_b = 1;
+    double best = 1e300;
+    const int bmax = a.Ho < 512 ? a.Ho : 512;
+    for (int b = 1; b <= bmax; ++b) {
+      const int h = ceil_div(a.Ho, b);
+      const int nb = ceil_div(a.Ho, h);  // bands actually used with height h
+      long long nbp = nb;
+      while ((static_cast<long long>(a.n_cb) * nbp) % kCtaWarps) ++nbp;
+      const long long ctas = groups * a.n_cb * nbp / kCtaWarps;
+      const long long waves = (ctas + resident_ctas - 1) / resident_ctas;
+      const double cost = static_cast<double>(waves) * (h + K - 1) * (1.0 + 1e-3 * (nbp - nb));
+      if (cost < best - 1e-9) {
+        best = cost;
+        best_b = nb;
+      }
+    }
+    band_h = ceil_div(a.Ho, best_b);
   }
   if (band_h > a.Ho) band_h = a.Ho;
   a.band_h = band_h;
