@@ -68,14 +68,17 @@ def fp32_fma_peak_tflops(sm_mhz):
 class Point:
     """One conv call of a step: shapes, device buffers, algorithmic work."""
 
-    def __init__(self, kind, name, dims, K):
+    def __init__(self, kind, name, dims, K, padding="valid", flip=False, halo_rows=0):
         self.kind, self.name, self.dims, self.K = kind, name, dims, K
-        self.x = self.f = self.y = None
+        self.padding, self.flip, self.halo_rows = padding, flip, halo_rows  # N4 / N3 variants (single)
+        self.x = self.f = self.y = self.halo = None
 
     @property
     def out_px(self):
         if self.kind == "single":
             H, W = self.dims
+            if self.padding != "valid":
+                return H * W
             return (H - self.K + 1) * (W - self.K + 1)
         N, C, H, W, F = self.dims
         return N * F * (H - self.K + 1) * (W - self.K + 1)
@@ -123,6 +126,12 @@ def workload_points(name):
         return [Point("multi", "N128 C3 F64 224^2 K7", (128, 3, 224, 224, 64), 7)], "GFLOP/s"
     if name == "config4":
         return [Point("single", "32768^2 K=15", (32768, 32768), 15)], "Gpixel/s"
+    if name == "pad":  # 'same' padding and true convolution
+        return [Point("single", f"8192^2 K={K} {pad}{' flip' if flip else ''}", (8192, 8192), K, pad, flip)
+                for K in (3, 15) for pad, flip in (("same_zero", False), ("same_replicate", True))], "Gpixel/s"
+    if name == "halo":  # the last K-1 rows read in place from a separate allocation
+        return [Point("single", f"8192^2 K={K} halo {K - 1} rows", (8192, 8192), K, halo_rows=K - 1)
+                for K in (3, 15)], "Gpixel/s"
     if name == "table1":  # PAPER.md Table I: 11 layers x C in {1, 3}, N = 128
         return [Point("multi", f"{nm} C{C} N128 {S}^2 F{F} K{K}", (128, C, S, S, F), K)
                 for C in (1, 3) for nm, S, F, K in TABLE1], "GFLOP/s"
@@ -142,6 +151,10 @@ WORKLOAD_DESC = {
     "config3": "BASELINE.json configs[3]: N=128, C=3, F=64, 224x224, K=7",
     "config4": "BASELINE.json configs[4]: 32768x32768, K=15 (row bands + NCCL halo at N>1)",
     "table1": "PAPER.md Table I (P:335-352): 11 layers x C in {1,3}, N=128 (22 conv2d_multi calls per step)",
+    "pad": "SURVEY 8(f) N4: 8192^2, K in {3,15}, 'same' zero padding / 'same' replicate padding + true "
+           "convolution (conv2d_single_pad; 4 calls per step)",
+    "halo": "SURVEY 8(f) N3: 8192^2, K in {3,15}, last K-1 rows in a separate allocation read in place "
+            "(conv2d_single_halo, the fused row-band halo launch on one GPU; 2 calls per step)",
 }
 
 
@@ -154,9 +167,14 @@ def materialise(points, rank, world, device):
         seed = synth.BASE_SEED + 1000 * rank + i
         if p.kind == "single":
             H, W = p.dims
-            p.x = synth.fill_torch(seed, synth.TAG_INPUT, (H, W), "img", device=device)
+            full = synth.fill_torch(seed, synth.TAG_INPUT, (H, W), "img", device=device)
+            hr = p.halo_rows
+            p.x = full[:H - hr].clone() if hr else full
+            p.halo = full[H - hr:].clone() if hr else None
+            del full
             p.f = torch.from_numpy(synth.make_filter(seed, p.K, "rand")[0, 0]).to(device)
-            p.y = torch.empty((H - p.K + 1, W - p.K + 1), device=device)
+            p.y = (torch.empty((H, W), device=device) if p.padding != "valid" else
+                   torch.empty((H - p.K + 1, W - p.K + 1), device=device))
         else:
             N, C, H, W, F = p.dims
             p.x = synth.fill_torch(seed, synth.TAG_INPUT, (N, C, H, W), "img" if C < 8 else "sym",
@@ -285,6 +303,10 @@ def run_ours(args):
             shard.rowband_conv2d_single_p2p(p.x, peer, p.f, band, p.y)
         elif rowband:
             shard.rowband_conv2d_single(p.x, p.f, band, p.y)
+        elif p.kind == "single" and p.halo is not None:
+            pkg.conv2d_single_halo(p.x, p.halo, p.f, out=p.y, stream=st)
+        elif p.kind == "single" and (p.padding != "valid" or p.flip):
+            pkg.conv2d_single_pad(p.x, p.f, p.padding, p.flip, out=p.y, stream=st)
         elif p.kind == "single":
             pkg.conv2d_single(p.x, p.f, out=p.y, stream=st)
         elif args.multi_impl == "tc":
@@ -572,9 +594,12 @@ def _oracle_sample(points, frac):
             x = synth.fill_np(seed, synth.TAG_INPUT, (rows + p.K - 1, W), "img")
             f = synth.make_filter(seed, p.K, "rand")[0, 0]
             t0 = time.perf_counter()
-            oracle.conv2d_single(x, f, want_bound=False)
+            if p.padding != "valid" or p.flip:
+                y, _, _ = oracle.conv2d_single_pad(x, f, p.padding, p.flip)
+            else:
+                y, _, _ = oracle.conv2d_single(x, f, want_bound=False)
             secs += time.perf_counter() - t0
-            units += rows * (W - p.K + 1)
+            units += y.size
         else:
             N, C, H, W, F = p.dims
             imgs = max(1, math.ceil(frac * N))
@@ -675,6 +700,8 @@ def main():
     args = ap.parse_args()
     if args.warmup < 3 and args.impl == "ours":
         args.warmup = 3  # contract: W >= 3
+    if args.workload in ("pad", "halo"):
+        args.no_e2e = True  # the host-buffer entry (e2e) is the valid-mode one-segment call
     if args.impl == "reference":
         run_reference(args)
     else:

@@ -213,6 +213,53 @@ int launch_split_v(const float *in, int H, int W, const float *filt, float *out,
   return with_const_filter(filt, K, KCfg<K>::KP, stream, go);
 }
 
+// The tuned default kernel choice (HALO: conv2d_single_halo's two-segment row addressing, same choice
+// and so the same bits as the one-segment call on the concatenated rows).
+template <int K, bool HALO>
+int launch_single_default(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream,
+                          int band_h, const DevInfo &dev, const float *in2, int H1, long long P, int min_band,
+                          bool constant_ok) {
+#define C2D_LS(UU, FS, PFF, G) \
+  launch_single_v<K, UU, FS, PFF, G, HALO>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1, P)
+#define C2D_SP(GG, UU, PFF, RR, CLL) \
+  launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(in, H, W, filt, out, stream, band_h, dev, 1, in2, H1, P)
+  // Narrow images with large K (latency regime: a full wave of one-warp tiles leaves bands of a few
+  // rows, and the K-1 prologue rows of Alg. 2 case 1 dominate): filter rows split over a cluster of 2
+  // one-warp CTAs (tools/split_sweep.py: 1024^2 K=15 24 -> 30 Gpx/s, 256^2 K=15 1.6 -> 3.8).
+  // Keyed on (W, K) only, so row bands of one image (same W) take the same kernel: bitwise seams.
+  if constexpr (K >= 11) {
+    if (constant_ok && W <= 1024) return C2D_SP(2, 1, 4, 4, 1);
+  }
+#undef C2D_SP
+  // Tuned on B200 (tools/variants.py sweeps, DESIGN.md "Kernel selection"):
+  //   K <= 5        two 128-column chunks per warp; row fetch from a 4-stage cp.async ring, except
+  //                 K <= 3 on wide images (one register row in flight is enough when HBM-bound);
+  //   K = 6..9      wide images (W >= 8192): two chunks + ring; narrower: one chunk + ring with
+  //                 Alg. 2 case-1/3 guards (short bands);
+  //   K = 10, 11    one chunk + ring + guards;
+  //   K >= 12       one chunk, register row fetch, guarded prologue on wide images (tall bands),
+  //                 guarded prologue + epilogue on narrow ones.
+  // Small images with K < 11 are latency-bound (a few microseconds): the per-CTA shared-memory filter
+  // skips the constant-slot staging (a stream-ordered copy plus two event operations, ~3 us of host
+  // and device time per call, tools/host_overhead.py). Same summation order, same bits.
+  const bool small = static_cast<long long>(H) * W <= 512LL * 512;
+  if (!constant_ok || (K < 11 && small))
+    return (K <= 7) ? C2D_LS(2, FSRC_SMEM, 1, 0) : C2D_LS(1, FSRC_SMEM, 1, 0);
+  if constexpr (K <= 5) {
+    if (K <= 3 && W > 1024) return C2D_LS(2, FSRC_CONST, 1, 0);
+    return C2D_LS(2, FSRC_CONST, 4, 0);
+  } else if constexpr (K <= 9) {
+    if (W >= 8192) return C2D_LS(2, FSRC_CONST, 4, 0);
+    return C2D_LS(1, FSRC_CONST, 4, 2);
+  } else if constexpr (K <= 11) {
+    return C2D_LS(1, FSRC_CONST, 4, 2);
+  } else {
+    if (W >= 4096) return C2D_LS(1, FSRC_CONST, 1, 1);
+    return C2D_LS(1, FSRC_CONST, 1, 2);
+  }
+#undef C2D_LS
+}
+
 template <int K>
 int launch_single(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
                   const DevInfo &dev, const float *in2, int H1, long long P) {
@@ -221,17 +268,8 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
   const int v = g_variant.load(std::memory_order_relaxed);
   // CUDA-graph capture cannot use the event-guarded constant slots: shared-memory filter there
   const bool constant_ok = !stream_capturing(stream);
-  if (H1 < H) {
-    // conv2d_single_halo: the halo instantiations (same sums as every one-tile variant: same bits),
-    // or the split kernel where the default takes it (it addresses both segments natively)
-    if constexpr (K >= 11) {
-      if (constant_ok && W <= 1024) return launch_split_v<K, 2, 1, 4, 4, 1, 1>(in, H, W, filt, out, stream, band_h,
-                                                                                 dev, 1, in2, H1, P);
-    }
-    if (!constant_ok)
-      return launch_single_v<K, 1, FSRC_SMEM, 1, 0, true>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1, P);
-    return launch_single_v<K, 1, FSRC_CONST, 4, 2, true>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1, P);
-  }
+  if (H1 < H) return launch_single_default<K, true>(in, H, W, filt, out, stream, band_h, dev, in2, H1, P, min_band,
+                                                    constant_ok);
 #define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1, P)
   switch (v) {
     case 1: return C2D_LS(1, FSRC_SMEM, 1, 0);
@@ -258,40 +296,7 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
       }
     }
   }
-  // Narrow images with large K (latency regime: a full wave of one-warp tiles leaves bands of a few
-  // rows, and the K-1 prologue rows of Alg. 2 case 1 dominate): filter rows split over a cluster of 2
-  // one-warp CTAs (tools/split_sweep.py: 1024^2 K=15 24 -> 30 Gpx/s, 256^2 K=15 1.6 -> 3.8).
-  // Keyed on (W, K) only, so row bands of one image (same W) take the same kernel: bitwise seams.
-  if constexpr (K >= 11) {
-    if (constant_ok && v == 0 && W <= 1024) return C2D_SP(2, 1, 4, 4, 1);
-  }
-#undef C2D_SP
-  // Tuned on B200 (tools/variants.py sweeps, DESIGN.md "Kernel selection"):
-  //   K <= 5        two 128-column chunks per warp; row fetch from a 4-stage cp.async ring, except
-  //                 K <= 3 on wide images (one register row in flight is enough when HBM-bound);
-  //   K = 6..9      wide images (W >= 8192): two chunks + ring; narrower: one chunk + ring with
-  //                 Alg. 2 case-1/3 guards (short bands);
-  //   K = 10, 11    one chunk + ring + guards;
-  //   K >= 12       one chunk, register row fetch, guarded prologue on wide images (tall bands),
-  //                 guarded prologue + epilogue on narrow ones.
-  // Small images with K < 11 are latency-bound (a few microseconds): the per-CTA shared-memory filter
-  // skips the constant-slot staging (a stream-ordered copy plus two event operations, ~3 us of host
-  // and device time per call, tools/host_overhead.py). Same summation order, same bits.
-  const bool small = static_cast<long long>(H) * W <= 512LL * 512;
-  if (!constant_ok || (K < 11 && small && v == 0))
-    return (K <= 7) ? C2D_LS(2, FSRC_SMEM, 1, 0) : C2D_LS(1, FSRC_SMEM, 1, 0);
-  if constexpr (K <= 5) {
-    if (K <= 3 && W > 1024) return C2D_LS(2, FSRC_CONST, 1, 0);
-    return C2D_LS(2, FSRC_CONST, 4, 0);
-  } else if constexpr (K <= 9) {
-    if (W >= 8192) return C2D_LS(2, FSRC_CONST, 4, 0);
-    return C2D_LS(1, FSRC_CONST, 4, 2);
-  } else if constexpr (K <= 11) {
-    return C2D_LS(1, FSRC_CONST, 4, 2);
-  } else {
-    if (W >= 4096) return C2D_LS(1, FSRC_CONST, 1, 1);
-    return C2D_LS(1, FSRC_CONST, 1, 2);
-  }
+  return launch_single_default<K, false>(in, H, W, filt, out, stream, band_h, dev, in2, H1, P, min_band, constant_ok);
 #undef C2D_LS
 }
 

@@ -13,7 +13,7 @@ fi
 timeout 900 python bench.py > gpurun_out/bench_$TAG.json 2> gpurun_out/bench_$TAG.err
 echo "bench rc=$?"
 if [ "${SKIP_WORKLOADS:-0}" != "1" ]; then
-  for wl in config0 config2 config3 config4 table1; do
+  for wl in config0 config2 config3 config4 table1 pad halo; do
     timeout 600 python bench.py --workload $wl --steps 10 > gpurun_out/bench_${TAG}_$wl.json 2> gpurun_out/bench_${TAG}_$wl.err
     echo "bench $wl rc=$?"
   done
@@ -27,7 +27,14 @@ fi
 timeout 900 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file gpurun_out/launches_$TAG.csv \
     python bench.py --steps 2 --warmup 3 --no-e2e --no-cpu-baseline > /dev/null 2>&1
 echo "ncu launches rc=$?"
-for spec in "15 0 8192" "3 0 8192"; do timeout 600 bash tools/prof2.sh "$spec" > /dev/null 2>&1; done
+for spec in "15 0 8192" "3 0 8192" "7 0 8192"; do timeout 600 bash tools/prof2.sh "$spec" > /dev/null 2>&1; done
+# the filter-row split kernel (default for W <= 1024, K >= 11) and the Table I CONV11 C1 multi kernel
+timeout 300 ncu --set full --clock-control none --import-source on -k regex:k_conv2d_split -s 3 -c 1 -o /tmp/prof_split \
+    python tools/prof_one.py single 1024 15 --reps 4 > /dev/null 2>&1
+ncu -i /tmp/prof_split.ncu-rep --page raw --csv > gpurun_out/prof_split_k15_s1024.raw.csv 2>/dev/null
+timeout 300 ncu --set full --clock-control none --import-source on -k regex:k_conv2d_multi -s 1 -c 1 -o /tmp/prof_conv11c1 \
+    python tools/prof_one.py multi 128,1,224,224,64 3 --reps 2 > /dev/null 2>&1
+ncu -i /tmp/prof_conv11c1.ncu-rep --page raw --csv > gpurun_out/prof_conv11c1.raw.csv 2>/dev/null
 timeout 300 ncu --set full --clock-control none -k regex:k_conv2d_direct -s 3 -c 1 -o /tmp/prof_direct \
     python tools/prof_one.py single 8192 3 --reps 4 --direct > /dev/null 2>&1
 ncu -i /tmp/prof_direct.ncu-rep --page raw --csv > gpurun_out/prof_direct_k3_s8192.raw.csv 2>/dev/null

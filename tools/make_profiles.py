@@ -28,6 +28,9 @@ CAPTURES = {
     "prof_direct_k3_s8192": "conv2d_single_direct 8192^2 K=3 (Fig. 1a baseline)",
     "prof_tc_config2": "conv2d_multi_tc N32 C64 F64 56^2 K3",
     "prof_tc_config3": "conv2d_multi_tc N128 C3 F64 224^2 K7",
+    "prof_k7_v0_s8192": "conv2d_single 8192^2 K=7",
+    "prof_split_k15_s1024": "conv2d_single 1024^2 K=15 (filter-row split, cluster of 2 CTAs)",
+    "prof_conv11c1": "conv2d_multi Table I CONV11 C1 N128 224^2 F64 K3",
 }
 
 
