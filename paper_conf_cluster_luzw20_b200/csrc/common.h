@@ -27,11 +27,16 @@ extern std::atomic<int> g_mvariant;   // multi-channel kernel variant
 cudaError_t scratch_alloc(void **p, size_t bytes, cudaStream_t stream);
 cudaError_t scratch_trim();
 
+// band_h value for single_entry: automatic band height, and never the filter-row split kernel (its
+// sums are grouped differently; conv2d_single_pad's border strips must match the one-tile kernel bits)
+constexpr int kBandNoSplit = -2;
+
 // per-K entry points, explicitly instantiated one K per translation unit (csrc/inst_kNN.cu)
 template <int K>
 int single_entry(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
                  const DevInfo &dev, const float *in2, int H1,
-                 long long P);  // rows >= H1 at in2 (H1 == H: one segment); input row pitch P floats
+                 long long P, int Po);  // rows >= H1 at in2 (H1 == H: one segment); input / output row
+                                        // pitch P / Po floats
 template <int K>
 int multi_entry(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
                 cudaStream_t stream, int band_h, const DevInfo &dev);

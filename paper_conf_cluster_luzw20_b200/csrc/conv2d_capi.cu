@@ -144,7 +144,7 @@ int conv2d_single_ex(const float *in, int H, int W, const float *filt, int K, fl
   DevInfo dev;
   if (current_device_info(&dev)) return CONV2D_ECUDA;
   cudaStream_t s = static_cast<cudaStream_t>(stream);
-#define C2D_CALL_SINGLE(KK) single_entry<KK>(in, H, W, filt, out, s, band_h, dev, in, H, W)
+#define C2D_CALL_SINGLE(KK) single_entry<KK>(in, H, W, filt, out, s, band_h, dev, in, H, W, W - KK + 1)
   C2D_K_SWITCH(K, C2D_CALL_SINGLE)
 #undef C2D_CALL_SINGLE
 }
@@ -169,7 +169,7 @@ int conv2d_single_halo(const float *in, int H, int W, const float *halo, int hal
   if (current_device_info(&dev)) return CONV2D_ECUDA;
   cudaStream_t s = static_cast<cudaStream_t>(stream);
   const int Hi = static_cast<int>(Ht);
-#define C2D_CALL_HALO(KK) single_entry<KK>(in, Hi, W, filt, out, s, 0, dev, halo, H, W)
+#define C2D_CALL_HALO(KK) single_entry<KK>(in, Hi, W, filt, out, s, 0, dev, halo, H, W, W - KK + 1)
   C2D_K_SWITCH(K, C2D_CALL_HALO)
 #undef C2D_CALL_HALO
 }

@@ -348,6 +348,7 @@ struct SingleArgs {
   int H1;            // rows [0, H1) at in, rows [H1, H) at in2 (H1 == H: one segment)
   int P;             // input row pitch in floats (>= W; == W for the C-ABI calls, padded buffers: % 4 == 0)
   int Wc;            // row-fetch bound: W, or P for a padded buffer (clamped quads stay in the pitch)
+  int Po;            // output row pitch in floats (>= Wo; == Wo for the C-ABI calls)
   const float *filt;
   float *out;
   int H, W, Ho, Wo;
@@ -367,7 +368,7 @@ __device__ __forceinline__ const float *in_row(const SingleArgs &a, int r) {
     return a.in + static_cast<size_t>(r) * a.P;
 }
 __device__ __forceinline__ float *out_row(const SingleArgs &a, int o) {
-  return a.out + static_cast<size_t>(o) * a.Wo;
+  return a.out + static_cast<size_t>(o) * a.Po;
 }
 
 // One warp tile: 128*U columns x output rows [ob, oe). Input rows [ob, oe+K-1) stream through once,

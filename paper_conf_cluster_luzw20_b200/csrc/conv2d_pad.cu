@@ -3,14 +3,14 @@
 //
 // Both reduce to the valid-mode, stride-1 cross-correlation the paper's kernels compute (PAPER.md
 // P:83-85; R1/R2): true convolution is cross-correlation with the filter rotated
-// by 180 degrees, and 'same' is the valid result on the image padded by K-1 rows and columns
+// by 180 degrees, and 'same' is the valid result on the image extended by K-1 rows and columns
 // (top/left (K-1)/2, bottom/right K-1-(K-1)/2, the convention of torch.nn.functional.conv2d
-// padding='same'). The rotation and the padding are pure data movement done by two small kernels
-// into the library's stream-ordered scratch pool; the padded image gets a 16-byte row pitch so the
-// convolution takes the vectorised row-fetch path; then the same per-K kernels as conv2d_single run
-// on it. Results are therefore bitwise equal to conv2d_single on the padded image / rotated filter.
-// (In-kernel padding would save the extra pass over the image -- ~2x traffic at HBM-bound K = 3 and
-// a few percent at FMA-bound K -- at the cost of another edge path through the hot kernels.)
+// padding='same'). The rotation is a one-block kernel into the library's stream-ordered scratch
+// pool. 'same' is computed as the interior -- one valid launch straight on the image, writing into
+// the output with its row pitch (no extra pass over the image) -- plus four thin border strips whose
+// slices of the extended image a small kernel materialises (16-byte row pitch) in the scratch pool.
+// Every launch is the same per-K one-tile kernels (never the filter-row split), so the result is
+// bitwise equal to the one-tile kernels on the fully padded image with the rotated filter.
 #include <cstdint>
 
 #include <cuda_runtime.h>
@@ -26,20 +26,20 @@ using namespace c2d;
 // input row r - pt; out-of-range entries are 0 (ZERO) or the nearest edge element (REPLICATE);
 // columns >= Wt (the pitch slack) are 0.
 __global__ void k_pad_image(const float *__restrict__ in, int H, int W, float *__restrict__ P, int Hp, int Wt,
-                            long long P4, int pt, int pl, int replicate) {
+                            long long P4, int pt, int pl, int replicate, int er0, int ec0) {
   const long long total = static_cast<long long>(Hp) * P4;
   for (long long q = static_cast<long long>(blockIdx.x) * blockDim.x + threadIdx.x; q < total;
        q += static_cast<long long>(gridDim.x) * blockDim.x) {
     const int r = static_cast<int>(q / P4);
     const int c0 = static_cast<int>(q % P4) * 4;
-    int ri = r - pt;
+    int ri = er0 + r - pt;  // (er0, ec0): this buffer's origin in the extended image
     const bool row_in = ri >= 0 && ri < H;
     if (replicate) ri = min(max(ri, 0), H - 1);
     float v[4];
 #pragma unroll
     for (int t = 0; t < 4; ++t) {
       const int c = c0 + t;
-      int ci = c - pl;
+      int ci = ec0 + c - pl;
       const bool col_in = ci >= 0 && ci < W;
       if (replicate) ci = min(max(ci, 0), W - 1);
       const bool take = c < Wt && (replicate || (row_in && col_in));
@@ -106,53 +106,79 @@ extern "C" int conv2d_single_pad(const float *in, int H, int W, const float *fil
     }
     f_use = f_rot;
   }
-  const float *src = in;
-  long long pitch = W;
-  float *padded = nullptr;
-  if (pad) {
-    pitch = (Wt + 3) / 4 * 4;  // 16-byte rows: the vectorised row fetch
-    const size_t p_b = static_cast<size_t>(Ht) * pitch * sizeof(float);
-    if (scratch_alloc(reinterpret_cast<void **>(&padded), p_b, s) != cudaSuccess) {
-      if (f_rot) cudaFreeAsync(f_rot, s);
-      return CONV2D_EALLOC;
+  // One valid-mode launch of the per-K kernels: `src` (rows x cols, row pitch `pitch`) into `dst`
+  // (output row pitch `po`). kBandNoSplit: the one-tile kernels everywhere in the padded call, so
+  // interior and border outputs sum in the same order whatever the strip widths.
+  auto conv = [&](const float *src, int rows, int cols, long long pitch, float *dst, int po) -> int {
+    switch (K) {
+#define C2D_CALL_PAD(KK) \
+  case KK: return single_entry<KK>(src, rows, cols, f_use, dst, s, kBandNoSplit, dev, src, rows, pitch, po);
+      C2D_CALL_PAD(1) C2D_CALL_PAD(2) C2D_CALL_PAD(3) C2D_CALL_PAD(4) C2D_CALL_PAD(5) C2D_CALL_PAD(6)
+      C2D_CALL_PAD(7) C2D_CALL_PAD(8) C2D_CALL_PAD(9) C2D_CALL_PAD(10) C2D_CALL_PAD(11) C2D_CALL_PAD(12)
+      C2D_CALL_PAD(13) C2D_CALL_PAD(14) C2D_CALL_PAD(15)
+#undef C2D_CALL_PAD
+      default: return CONV2D_EK;
     }
-    const long long quads = Ht * (pitch / 4);
+  };
+  if (!pad) {
+    const int rc = conv(in, H, W, W, out, W - K + 1);
+    if (f_rot) cudaFreeAsync(f_rot, s);
+    return rc;
+  }
+  // 'same': out (H x W) = valid correlation of the extended image E ((H+K-1) x (W+K-1)). The interior
+  // [pt, pt+H-K+1) x [pl, pl+W-K+1) reads only the image itself: one launch straight on `in`, writing
+  // into `out` with row pitch W -- no extra pass over the image. The four border strips (top pt rows,
+  // bottom pb rows, left pl / right pr columns of the rows between) each read a thin slice of E, which
+  // k_pad_image materialises (16-byte pitch) in the scratch pool. Images smaller than the filter,
+  // and K >= 9: all of E at once.
+  const int pt = (K - 1) / 2, pb = K - 1 - pt, pl = pt, pr = pb;
+  struct Strip {
+    int er0, ec0, rows, cols;  // slice of E
+    long long out_off;         // first output element
+  };
+  Strip strips[5];
+  int ns = 0;
+  // K >= 9 (FMA-bound): the strips -- latency-bound launches on images a few rows or columns wide --
+  // cost more than one extra pass over the image (8192^2 K=15: 0.70 vs 0.67 ms), so E is padded whole;
+  // K < 9 (HBM-bound): interior + strips (8192^2 K=3: 0.137 vs 0.197 ms). Same bits either way.
+  const bool interior = H >= K && W >= K && K < 9;
+  const int WE = W + K - 1;  // width of E
+  if (!interior) {
+    strips[ns++] = {0, 0, H + K - 1, WE, 0};
+  } else {
+    if (pt > 0) strips[ns++] = {0, 0, pt + K - 1, WE, 0};
+    if (pb > 0) strips[ns++] = {H - pb, 0, pb + K - 1, WE, static_cast<long long>(H - pb) * W};
+    if (pl > 0) strips[ns++] = {pt, 0, H, pl + K - 1, static_cast<long long>(pt) * W};
+    if (pr > 0) strips[ns++] = {pt, W - pr, H, pr + K - 1, static_cast<long long>(pt) * W + W - pr};
+  }
+  long long off[5], total = 0;
+  for (int t = 0; t < ns; ++t) {
+    off[t] = total;
+    const long long p4 = (strips[t].cols + 3) / 4 * 4;
+    total += static_cast<long long>(strips[t].rows) * p4 + 4;  // +4: keeps every strip 16-byte aligned
+  }
+  float *scratch = nullptr;
+  if (ns > 0 && scratch_alloc(reinterpret_cast<void **>(&scratch), static_cast<size_t>(total) * sizeof(float), s) !=
+                    cudaSuccess) {
+    if (f_rot) cudaFreeAsync(f_rot, s);
+    return CONV2D_EALLOC;
+  }
+  int rc = CONV2D_OK;
+  for (int t = 0; t < ns && rc == CONV2D_OK; ++t) {
+    const Strip &st = strips[t];
+    const long long p4 = (st.cols + 3) / 4 * 4;
+    float *buf = scratch + off[t];
+    const long long quads = static_cast<long long>(st.rows) * (p4 / 4);
     long long blocks = (quads + 255) / 256;
     const long long cap = static_cast<long long>(dev.num_sms) * 8;
     if (blocks > cap) blocks = cap;
-    k_pad_image<<<static_cast<unsigned>(blocks), 256, 0, s>>>(in, H, W, padded, static_cast<int>(Ht),
-                                                              static_cast<int>(Wt), pitch / 4, (K - 1) / 2,
-                                                              (K - 1) / 2, pad == CONV2D_PAD_REPLICATE ? 1 : 0);
-    if (cudaGetLastError() != cudaSuccess) {
-      cudaFreeAsync(padded, s);
-      if (f_rot) cudaFreeAsync(f_rot, s);
-      return CONV2D_ECUDA;
-    }
-    src = padded;
+    k_pad_image<<<static_cast<unsigned>(blocks), 256, 0, s>>>(in, H, W, buf, st.rows, st.cols, p4 / 4, pt, pl,
+                                                              pad == CONV2D_PAD_REPLICATE ? 1 : 0, st.er0, st.ec0);
+    if (cudaGetLastError() != cudaSuccess) rc = CONV2D_ECUDA;
+    if (rc == CONV2D_OK) rc = conv(buf, st.rows, st.cols, p4, out + st.out_off, W);
   }
-  const int Hi = static_cast<int>(Ht), Wi = static_cast<int>(Wt);
-  int rc;
-#define C2D_CALL_PAD(KK) rc = single_entry<KK>(src, Hi, Wi, f_use, out, s, 0, dev, src, Hi, pitch); break;
-  switch (K) {
-    case 1: C2D_CALL_PAD(1)
-    case 2: C2D_CALL_PAD(2)
-    case 3: C2D_CALL_PAD(3)
-    case 4: C2D_CALL_PAD(4)
-    case 5: C2D_CALL_PAD(5)
-    case 6: C2D_CALL_PAD(6)
-    case 7: C2D_CALL_PAD(7)
-    case 8: C2D_CALL_PAD(8)
-    case 9: C2D_CALL_PAD(9)
-    case 10: C2D_CALL_PAD(10)
-    case 11: C2D_CALL_PAD(11)
-    case 12: C2D_CALL_PAD(12)
-    case 13: C2D_CALL_PAD(13)
-    case 14: C2D_CALL_PAD(14)
-    default: C2D_CALL_PAD(15)
-  }
-#undef C2D_CALL_PAD
-  // scratch returns to the pool once the convolution (ordered before on s) has read it
-  if (padded) cudaFreeAsync(padded, s);
+  if (rc == CONV2D_OK && interior) rc = conv(in, H, W, W, out + static_cast<long long>(pt) * W + pl, W);
+  if (scratch) cudaFreeAsync(scratch, s);
   if (f_rot) cudaFreeAsync(f_rot, s);
   return rc;
 }

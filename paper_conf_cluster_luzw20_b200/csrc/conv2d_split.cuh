@@ -36,6 +36,7 @@ struct SplitArgs {
   int H1;
   int P;        // input row pitch in floats, as SingleArgs
   int Wc;       // row-fetch bound, as SingleArgs
+  int Po;       // output row pitch, as SingleArgs
   float *out;
   int H, W, Ho, Wo;
   int band_h;   // output rows per cluster tile
@@ -220,7 +221,7 @@ __device__ __forceinline__ void split_tile(const SplitArgs &a, const FilterSrc<K
           }
         }
       }
-      float *orow = a.out + static_cast<size_t>(ob + c * R + k) * a.Wo;
+      float *orow = a.out + static_cast<size_t>(ob + c * R + k) * a.Po;
       store_row<U, SAFE>(orow, x0, a.Wo, o, lane);
     }
   };

@@ -3,7 +3,7 @@
 
 namespace c2d {
 template int single_entry<6>(const float *, int, int, const float *, float *, cudaStream_t, int, const DevInfo &,
-                                   const float *, int, long long);
+                                   const float *, int, long long, int);
 template int multi_entry<6>(const float *, int, int, int, int, const float *, int, float *, cudaStream_t, int,
                              const DevInfo &);
 }  // namespace c2d

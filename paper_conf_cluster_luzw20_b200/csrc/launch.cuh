@@ -92,7 +92,7 @@ bool stream_capturing(cudaStream_t s) {
 
 template <int K, int U, int FSRC, int PF = 1, int GUARDS = 0, bool HALO = false>
 int launch_single_v(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                    const DevInfo &dev, int min_band, const float *in2, int H1, long long P) {
+                    const DevInfo &dev, int min_band, const float *in2, int H1, long long P, int Po) {
   constexpr int CTAW = (FSRC == FSRC_CONST) ? 1 : kCtaWarps;
   auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS, HALO>;
   static std::atomic<int> occ_cache{0};
@@ -103,6 +103,7 @@ int launch_single_v(const float *in, int H, int W, const float *filt, float *out
   a.H1 = H1;
   a.P = static_cast<int>(P);
   a.Wc = static_cast<int>(P);
+  a.Po = Po;
   a.filt = filt;
   a.out = out;
   a.H = H;
@@ -137,7 +138,7 @@ int launch_single_v(const float *in, int H, int W, const float *filt, float *out
 // G times fewer, taller bands.
 template <int K, int G, int U, int PF, int R, int GUARDS, int CL>
 int launch_split_v(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                   const DevInfo &dev, int min_band, const float *in2, int H1, long long P) {
+                   const DevInfo &dev, int min_band, const float *in2, int H1, long long P, int Po) {
   static_assert(G >= 1 && G <= 8 && G <= K, "portable cluster of at most K CTAs");
   auto kernel = k_conv2d_split<K, G, U, PF, R, GUARDS, CL>;
   static std::atomic<int> occ_cache{0};
@@ -149,6 +150,7 @@ int launch_split_v(const float *in, int H, int W, const float *filt, float *out,
   a.H1 = H1;
   a.P = static_cast<int>(P);
   a.Wc = static_cast<int>(P);
+  a.Po = Po;
   a.out = out;
   a.H = H;
   a.W = W;
@@ -217,18 +219,20 @@ int launch_split_v(const float *in, int H, int W, const float *filt, float *out,
 // and so the same bits as the one-segment call on the concatenated rows).
 template <int K, bool HALO>
 int launch_single_default(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream,
-                          int band_h, const DevInfo &dev, const float *in2, int H1, long long P, int min_band,
-                          bool constant_ok) {
+                          int band_h, const DevInfo &dev, const float *in2, int H1, long long P, int Po,
+                          int min_band, bool constant_ok) {
 #define C2D_LS(UU, FS, PFF, G) \
-  launch_single_v<K, UU, FS, PFF, G, HALO>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1, P)
+  launch_single_v<K, UU, FS, PFF, G, HALO>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1, P, Po)
 #define C2D_SP(GG, UU, PFF, RR, CLL) \
-  launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(in, H, W, filt, out, stream, band_h, dev, 1, in2, H1, P)
+  launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(in, H, W, filt, out, stream, band_h, dev, 1, in2, H1, P, Po)
+  const bool no_split = band_h == kBandNoSplit;  // internal callers that need the one-tile kernel's bits
+  if (no_split) band_h = 0;
   // Narrow images with large K (latency regime: a full wave of one-warp tiles leaves bands of a few
   // rows, and the K-1 prologue rows of Alg. 2 case 1 dominate): filter rows split over a cluster of 2
   // one-warp CTAs (tools/split_sweep.py: 1024^2 K=15 24 -> 30 Gpx/s, 256^2 K=15 1.6 -> 3.8).
   // Keyed on (W, K) only, so row bands of one image (same W) take the same kernel: bitwise seams.
   if constexpr (K >= 11) {
-    if (constant_ok && W <= 1024) return C2D_SP(2, 1, 4, 4, 1);
+    if (constant_ok && W <= 1024 && !no_split) return C2D_SP(2, 1, 4, 4, 1);
   }
 #undef C2D_SP
   // Tuned on B200 (tools/variants.py sweeps):
@@ -262,15 +266,15 @@ int launch_single_default(const float *in, int H, int W, const float *filt, floa
 
 template <int K>
 int launch_single(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                  const DevInfo &dev, const float *in2, int H1, long long P) {
+                  const DevInfo &dev, const float *in2, int H1, long long P, int Po) {
   const int mb = g_min_band.load(std::memory_order_relaxed);
   const int min_band = mb > 0 ? mb : (K - 1 > 4 ? K - 1 : 4);
   const int v = g_variant.load(std::memory_order_relaxed);
   // CUDA-graph capture cannot use the event-guarded constant slots: shared-memory filter there
   const bool constant_ok = !stream_capturing(stream);
-  if (H1 < H) return launch_single_default<K, true>(in, H, W, filt, out, stream, band_h, dev, in2, H1, P, min_band,
+  if (H1 < H) return launch_single_default<K, true>(in, H, W, filt, out, stream, band_h, dev, in2, H1, P, Po, min_band,
                                                     constant_ok);
-#define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1, P)
+#define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1, P, Po)
   switch (v) {
     case 1: return C2D_LS(1, FSRC_SMEM, 1, 0);
     case 2: return C2D_LS(2, FSRC_SMEM, 1, 0);
@@ -285,7 +289,7 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
   }
   // filter-row split (conv2d_split.cuh; variants 10-12)
 #define C2D_SP(GG, UU, PFF, RR, CLL) \
-  launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(in, H, W, filt, out, stream, band_h, dev, 1, in2, H1, P)
+  launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(in, H, W, filt, out, stream, band_h, dev, 1, in2, H1, P, Po)
   if (constant_ok && v >= 10 && v <= 12) {
     if constexpr (K >= 3) {
       switch (v) {
@@ -296,7 +300,8 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
       }
     }
   }
-  return launch_single_default<K, false>(in, H, W, filt, out, stream, band_h, dev, in2, H1, P, min_band, constant_ok);
+  return launch_single_default<K, false>(in, H, W, filt, out, stream, band_h, dev, in2, H1, P, Po, min_band,
+                                         constant_ok);
 #undef C2D_LS
 }
 
@@ -492,8 +497,8 @@ namespace c2d {
 
 template <int K>
 int single_entry(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                 const DevInfo &dev, const float *in2, int H1, long long P) {
-  return launch_single<K>(in, H, W, filt, out, stream, band_h, dev, in2, H1, P);
+                 const DevInfo &dev, const float *in2, int H1, long long P, int Po) {
+  return launch_single<K>(in, H, W, filt, out, stream, band_h, dev, in2, H1, P, Po);
 }
 
 template <int K>

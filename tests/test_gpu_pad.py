@@ -47,18 +47,24 @@ def test_pad_integer_data_exact(cuda_device, K):
         _check(x, f, padding, flip, pkg.conv2d_single_pad(x, f, padding, flip), exact=True)
 
 
-@pytest.mark.parametrize("K", [3, 5, 15])
+@pytest.mark.parametrize("K", [2, 3, 5, 12, 15])
 def test_pad_is_conv2d_single_of_padded_image_bitwise(cuda_device, K):
-    """'same' = valid on the padded image, flip = rotated filter: the same kernels see the same data."""
+    """'same' = valid on the padded image, flip = rotated filter: interior launch + border strips give
+    the bits of one one-tile-kernel call on the fully padded image (variant 1 as the reference: the
+    default would take the filter-row split for narrow images with K >= 11)."""
     pt = (K - 1) // 2
     f = torch.from_numpy(synth.make_filter(K + 1, K, "rand")[0, 0]).to(DEV)
-    for (H, W) in [(200, 333), (K + 60, 2048)]:
+    for (H, W) in [(200, 333), (K + 60, 2048), (K - 1, 50), (7, K + 2)]:
         x = dev_image((H, W), "sym", seed=W + K)
         for mode in ("constant", "replicate"):
             xp = torch.nn.functional.pad(x[None, None], (pt, K - 1 - pt, pt, K - 1 - pt), mode=mode)[0, 0]
             for flip in (False, True):
                 g = torch.flip(f, (0, 1)) if flip else f
-                ref = pkg.conv2d_single(xp.contiguous(), g.contiguous())
+                _capi.debug_set_variant(1)
+                try:
+                    ref = pkg.conv2d_single(xp.contiguous(), g.contiguous())
+                finally:
+                    _capi.debug_set_variant(0)
                 got = pkg.conv2d_single_pad(x, f, "same_zero" if mode == "constant" else "same_replicate", flip)
                 torch.cuda.synchronize()
                 assert torch.equal(got, ref), (K, H, W, mode, flip)
