@@ -476,8 +476,13 @@ int launch_multi(const float *in, int N, int C, int H, int W, const float *filt,
   // ragged edge is a smaller share; FB = 8 filters per warp for K <= 3, half the register-limited FB
   // above (smaller loop body, more resident warps).
   const bool seg16 = (mv == 2 || mv == 4) || (mv == 0 && N >= 2 && lane_use(Wo, 64) >= lane_use(Wo, 128) - 0.05);
+  // 8-lane segments (four images per warp, 32 columns each) for narrow layers: Table I's 8-26-column
+  // outputs use 25-81% of the lanes instead of 12-41% (tools/multi_band_sweep.py)
+  const bool seg8 = mv == 7 || (mv == 0 && N >= 4 && Wo <= 32 && lane_use(Wo, 32) >= lane_use(Wo, 64) + 0.15);
   const bool half = (mv == 3 || mv == 4) || (mv == 0 && K > 3);
-  if (half)
+  if (seg8)
+    rc = half ? C2D_LM(FBH, 8) : C2D_LM(FB, 8);
+  else if (half)
     rc = seg16 ? C2D_LM(FBH, 16) : C2D_LM(FBH, 32);
   else
     rc = seg16 ? C2D_LM(FB, 16) : C2D_LM(FB, 32);

@@ -144,3 +144,25 @@ def test_tensor_core_variant_config3_sampled(cuda_device):
     ys = np.concatenate([rng.integers(0, Ho, P), np.array([0, Ho - 1] * 50)])
     xs = np.concatenate([rng.integers(0, Ho, P), np.array([Ho - 1, 0] * 50)])
     check_points_multi(x, w, y, rng.integers(0, N, len(ys)), rng.integers(0, F, len(ys)), ys, xs)
+
+
+@pytest.mark.parametrize("K", [1, 3, 5, 9, 15])
+def test_eight_lane_segments(cuda_device, K):
+    """8-lane segments (four images per warp, multi variant 7; the default for narrow layers): parity
+    with N not a multiple of 4, widths past one 32-column segment, integer data exact, band-split bits."""
+    from paper_conf_cluster_luzw20_b200 import _capi
+
+    try:
+        _capi.debug_set_multi_variant(7)
+        for (N, C, F, dh, dw) in [(5, 3, 9, 5, 7), (4, 1, 17, 12, 30), (2, 2, 3, 3, 40), (9, 1, 8, 1, 0)]:
+            x = dev_image((N, C, K + dh, K + dw), "img", seed=K + N)
+            w = _w(F, C, K, seed=K + F)
+            y = pkg.conv2d_multi(x, w)
+            check_full_multi(x, w, y)
+            for bh in (1, 4):
+                assert torch.equal(pkg.conv2d_multi(x, w, band_h=bh), y), (K, N, bh)
+        xi = dev_image((6, 3, K + 9, K + 20), "int", seed=K)
+        wi = _w(7, 3, K, "int", seed=K)
+        check_full_multi(xi, wi, pkg.conv2d_multi(xi, wi), exact=True)
+    finally:
+        _capi.debug_set_multi_variant(0)
