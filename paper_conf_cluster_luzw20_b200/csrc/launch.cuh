@@ -246,7 +246,9 @@ int launch_single_default(const float *in, int H, int W, const float *filt, floa
   // Small images with K < 11 are latency-bound (a few microseconds): the per-CTA shared-memory filter
   // skips the constant-slot staging (a stream-ordered copy plus two event operations, ~3 us of host
   // and device time per call, tools/host_overhead.py). Same summation order, same bits.
-  const bool small = static_cast<long long>(H) * W <= 512LL * 512;
+  // (tools/small_sizes2.py, back-to-back calls: 1024^2 K=3 12.1 -> 8.0 us, K=5 12.0 -> 10.3 us)
+  const long long px = static_cast<long long>(H) * W;
+  const bool small = px <= 512LL * 512 || (K <= 5 && px <= 1024LL * 1024);
   if (!constant_ok || (K < 11 && small))
     return (K <= 7) ? C2D_LS(2, FSRC_SMEM, 1, 0) : C2D_LS(1, FSRC_SMEM, 1, 0);
   if constexpr (K <= 5) {
