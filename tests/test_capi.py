@@ -82,6 +82,22 @@ def test_argument_errors_need_no_gpu(lib):
     assert c.conv2d_multi(a, 1, 1, 8, 8, b, 1, 16, o) == c.CONV2D_EK
     assert c.conv2d_multi(a, 2, 2, 8, 8, b, 1, 3, a + 100) == c.CONV2D_EOVERLAP
     assert c.conv2d_single_direct(a, 8, 8, b, 20, o) == c.CONV2D_EK
+    # conv2d_single_halo (N3): rows of `in` then rows of `halo`
+    h = 0x60000000
+    assert c.conv2d_single_halo(a, 8, 8, None, 2, b, 3, o) == c.CONV2D_ENULL
+    assert c.conv2d_single_halo(a, 8, 8, h, -1, b, 3, o) == c.CONV2D_ESHAPE
+    assert c.conv2d_single_halo(a, 8, 8, h, 2, b, 16, o) == c.CONV2D_EK
+    assert c.conv2d_single_halo(a, 1, 8, h, 1, b, 3, o) == c.CONV2D_ESHAPE  # 2 rows < K
+    assert c.conv2d_single_halo(a, 8, 8, h + 2, 2, b, 3, o) == c.CONV2D_EALIGN
+    assert c.conv2d_single_halo(a, 8, 8, h, 2, b, 3, h + 8) == c.CONV2D_EOVERLAP
+    # conv2d_single_pad (N4): mode bits, 'same' allows images smaller than the filter
+    assert c.conv2d_single_pad(a, 8, 8, b, 3, 3, o) == c.CONV2D_ESHAPE  # both PAD flags
+    assert c.conv2d_single_pad(a, 8, 8, b, 3, 8, o) == c.CONV2D_ESHAPE  # unknown bit
+    assert c.conv2d_single_pad(None, 8, 8, b, 3, 1, o) == c.CONV2D_ENULL
+    assert c.conv2d_single_pad(a, 8, 8, b, 16, 1, o) == c.CONV2D_EK
+    assert c.conv2d_single_pad(a, 2, 8, b, 3, c.CONV2D_FLIP, o) == c.CONV2D_ESHAPE  # valid needs H >= K
+    assert c.conv2d_single_pad(a, 0, 8, b, 3, 1, o) == c.CONV2D_ESHAPE
+    assert c.conv2d_single_pad(a, 8, 8, b, 3, 2, a + 32) == c.CONV2D_EOVERLAP
 
 
 def test_library_is_sm100a(lib):
