@@ -270,7 +270,12 @@ template <int K>
 int launch_single(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
                   const DevInfo &dev, const float *in2, int H1, long long P, int Po) {
   const int mb = g_min_band.load(std::memory_order_relaxed);
-  const int min_band = mb > 0 ? mb : (K - 1 > 4 ? K - 1 : 4);
+  // Minimum band height K-1 (>= 4) bounds the Alg. 2 case-1 overhead once a wave is full; images up
+  // to 512^2 cannot fill a wave even with one-row bands, and there the latency of a band's row chain
+  // dominates: no minimum (tools/latency.py, one 256^2 call: K=3 10.3 -> 8.9 us, K=9 20.7 -> 14.2 us,
+  // K=15 smem path 42 -> 28.6 us). Band height never changes the bits.
+  const bool tiny = static_cast<long long>(H) * W <= 512LL * 512;
+  const int min_band = mb > 0 ? mb : (tiny ? 1 : (K - 1 > 4 ? K - 1 : 4));
   const int v = g_variant.load(std::memory_order_relaxed);
   // CUDA-graph capture cannot use the event-guarded constant slots: shared-memory filter there
   const bool constant_ok = !stream_capturing(stream);
