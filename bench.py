@@ -273,15 +273,17 @@ def run_ours(args):
         peer = None
         if args.halo == "p2p":  # band buffers in symmetric memory: the halo is read in place over NVLink
             p.x, peer, p2p_handle = shard.symmetric_band_buffers(band, device)
+        elif args.halo == "ipc":  # same, buffers exchanged as CUDA IPC mappings (lazy peer access)
+            p.x, peer, p2p_keep = shard.ipc_band_buffers(band, device)
         else:
             p.x = torch.empty((band.buf_rows, W), device=device)
         p.x[:band.in_rows] = synth.fill_torch(synth.BASE_SEED, synth.TAG_INPUT, (band.in_rows, W), "img",
                                               start=band.o0 * W, device=device)
         p.f = torch.from_numpy(synth.make_filter(synth.BASE_SEED, p.K, "gauss")[0, 0]).to(device)
         p.y = torch.empty((band.out_rows, W - p.K + 1), device=device)
-        if args.halo == "p2p":  # every neighbour's rows are written before any rank reads them in place
+        if args.halo in ("p2p", "ipc"):  # every neighbour's rows are written before any rank reads them
             torch.cuda.synchronize()
-            p2p_handle.barrier()
+            dist.barrier()
     else:
         materialise(points, rank, world, device)
     stream = torch.cuda.current_stream(device)
@@ -299,7 +301,7 @@ def run_ours(args):
 
     def run_point(p):
         st = None if capturing[0] else stream  # under capture: torch's capture stream
-        if rowband and args.halo == "p2p":
+        if rowband and args.halo in ("p2p", "ipc"):
             shard.rowband_conv2d_single_p2p(p.x, peer, p.f, band, p.y)
         elif rowband:
             shard.rowband_conv2d_single(p.x, p.f, band, p.y)
@@ -448,7 +450,7 @@ def run_ours(args):
                    "l2": "512 MiB write + 256 MiB read between timed steps (outside the events) + distinct buffers per "
                          "conv; 8192^2 inputs also exceed L2",
                    "parallelism": (("row bands + NCCL halo" if args.halo == "nccl" else
-                                    "row bands, halo read in place from the neighbour (symmetric memory, NVLink)")
+                                    f"row bands, halo read in place from the neighbour ({args.halo}, NVLink)")
                                    if rowband else
                                    ("replicas (independent images per rank)" if world > 1 else "1 GPU")),
                    "filter": "rand (2u-1)/K", "input": "img u in [0,1)"},
@@ -691,8 +693,9 @@ def main():
     ap.add_argument("--cpu-budget", type=float, default=10.0)
     ap.add_argument("--ref-budget", type=float, default=90.0)
     ap.add_argument("--variant", type=int, default=0, help="tuning: force a single-channel kernel variant")
-    ap.add_argument("--halo", choices=["nccl", "p2p"], default="nccl",
-                    help="config4 at N>1: NCCL P2P halo exchange (+ tail call), or the fused in-place halo read")
+    ap.add_argument("--halo", choices=["nccl", "p2p", "ipc"], default="nccl",
+                    help="config4 at N>1: NCCL P2P halo exchange (+ tail call), or the fused in-place halo read "
+                         "from the neighbour's band mapped by symmetric memory (p2p) or CUDA IPC (ipc)")
     ap.add_argument("--graph", choices=["auto", "on", "off"], default="auto",
                     help="replay the step as a CUDA graph (auto: config0, the latency-bound single 256^2 call)")
     ap.add_argument("--multi-impl", choices=["cuda", "tc"], default="cuda",

@@ -156,6 +156,24 @@ def symmetric_band_buffers(band: RowBand, device, group=None):
     return buf, peer, handle
 
 
+def ipc_band_buffers(band: RowBand, device, group=None):
+    """Same contract as symmetric_band_buffers, transported by CUDA IPC: every rank allocates its band
+    buffer, the IPC handles are exchanged over the process group (all_gather_object), and rank p
+    opens rank p+1's buffer in its own address space (lazy peer access over NVLink when the ranks
+    are on different GPUs; a plain IPC mapping when they share one -- which lets one GPU test the
+    in-place halo path across processes). Returns (buf, peer_halo, keepalive)."""
+    from torch.multiprocessing.reductions import reduce_tensor
+
+    buf = torch.empty((band.in_rows, band.W), dtype=torch.float32, device=device)
+    handles = [None] * band.world
+    dist.all_gather_object(handles, reduce_tensor(buf), group=group)
+    peer = None
+    if not band.is_last and band.halo > 0:
+        rebuild, args = handles[band.rank + 1]
+        peer = rebuild(*args)[:band.halo]
+    return buf, peer, handles
+
+
 def rowband_conv2d_single_p2p(buf: torch.Tensor, peer_halo, f: torch.Tensor, band: RowBand, out: torch.Tensor,
                               compute_halo=_default_compute_halo, compute=_default_compute) -> torch.Tensor:
     """Row-band convolution with the halo read in place from the neighbour (one launch per rank).
