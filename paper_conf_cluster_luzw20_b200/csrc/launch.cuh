@@ -45,7 +45,7 @@ int cta_occupancy(KernelT kernel, size_t dyn_smem, std::atomic<int> &cache, int 
 // Variant override for tuning tools (c2d_debug_set_variant; 0 = the tuned default):
 //   1: filter in shared memory, U=1 (4 warps/CTA)     2: shared memory, U=2
 //   3: filter in a __constant__ slot, U=1 (1 warp/CTA) 4: __constant__ slot, U=2
-//   5-9: guard / prefetch variants of the constant-slot kernel (see launch_single)
+//   5-9, 13: guard / prefetch variants of the constant-slot kernel (see launch_single)
 //   10-12: filter-row split over G parts (conv2d_split.cuh)
 
 // Constant-bank filter slot of this unit (this K), per device: it holds the filter of the last call
@@ -254,6 +254,11 @@ int launch_single_default(const float *in, int H, int W, const float *filt, floa
   if constexpr (K <= 5) {
     if (K <= 3 && W > 1024) return C2D_LS(2, FSRC_CONST, 1, 0);
     return C2D_LS(2, FSRC_CONST, 4, 0);
+  } else if constexpr (K <= 7) {
+    // K = 6, 7: two chunks + ring with both Alg. 2 edge cases guarded on wide images
+    // (tools/split_sweep.py variant 14: 8192^2 K=7 445 -> 458 Gpx/s, 4096^2 333 -> 348)
+    if (W >= 4096) return C2D_LS(2, FSRC_CONST, 4, 2);
+    return C2D_LS(1, FSRC_CONST, 4, 2);
   } else if constexpr (K <= 9) {
     if (W >= 8192) return C2D_LS(2, FSRC_CONST, 4, 0);
     return C2D_LS(1, FSRC_CONST, 4, 2);
@@ -292,6 +297,7 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
     case 7: if (constant_ok) return C2D_LS(2, FSRC_CONST, 4, 0); break;
     case 8: if (constant_ok) return C2D_LS(2, FSRC_CONST, 8, 0); break;
     case 9: if (constant_ok) return C2D_LS(1, FSRC_CONST, 4, 2); break;
+    case 13: if constexpr (K >= 5 && K <= 9) { if (constant_ok) return C2D_LS(2, FSRC_CONST, 4, 2); } break;
     default: break;
   }
   // filter-row split (conv2d_split.cuh; variants 10-12)

@@ -168,7 +168,7 @@ def test_config4_32768_k15_sampled(cuda_device):
         assert torch.equal(part, y[lo:hi])
 
 
-@pytest.mark.parametrize("variant", [1, 2, 3, 4, 5, 6])
+@pytest.mark.parametrize("variant", [1, 2, 3, 4, 5, 6, 7, 9, 13])
 def test_every_kernel_variant_bitwise_equal(cuda_device, variant):
     """Every instantiation (filter in shared / constant memory, 1 or 2 column chunks, guarded or
     unguarded band prologue/epilogue) of the one-warp-tile kernel gives the same bits as variant 1,
