@@ -177,6 +177,8 @@ def test_every_kernel_variant_bitwise_equal(cuda_device, variant):
     shapes = [(40, 300), (77, 1030), (300, 517)]
     try:
         for K in (1, 2, 3, 5, 8, 9, 12, 15):
+            if variant == 13 and not 5 <= K <= 9:
+                continue  # variant 13 is instantiated for K = 5..9 only (elsewhere it means the default)
             f = _filt(K, "rand", seed=K)
             for (dh, W) in shapes:
                 x = dev_image((K + dh, W), "img", seed=K * 7 + W)
