@@ -30,6 +30,9 @@ cudaError_t scratch_trim();
 // band_h value for single_entry: automatic band height, and never the filter-row split kernel (its
 // sums are grouped differently; conv2d_single_pad's border strips must match the one-tile kernel bits)
 constexpr int kBandNoSplit = -2;
+// ... and with the per-CTA shared-memory filter (no constant-slot staging: a call on a side stream
+// must not wait for the slot's previous user on the main stream)
+constexpr int kBandSmemFilter = -3;
 
 // per-K entry points, explicitly instantiated one K per translation unit (csrc/inst_kNN.cu)
 template <int K>

@@ -8,10 +8,12 @@
 // padding='same'). The rotation is a one-block kernel into the library's stream-ordered scratch
 // pool. 'same' is computed as the interior -- one valid launch straight on the image, writing into
 // the output with its row pitch (no extra pass over the image) -- plus four thin border strips whose
-// slices of the extended image a small kernel materialises (16-byte row pitch) in the scratch pool.
+// slices of the extended image a small kernel materialises (16-byte row pitch) in the scratch pool,
+// on a side stream concurrent with the interior.
 // Every launch is the same per-K one-tile kernels (never the filter-row split), so the result is
 // bitwise equal to the one-tile kernels on the fully padded image with the rotated filter.
 #include <cstdint>
+#include <mutex>
 
 #include <cuda_runtime.h>
 
@@ -57,6 +59,20 @@ __global__ void k_rotate_filter(const float *__restrict__ f, int K, float *__res
 bool overlap(const void *a, size_t abytes, const void *b, size_t bbytes) {
   const uintptr_t a0 = reinterpret_cast<uintptr_t>(a), b0 = reinterpret_cast<uintptr_t>(b);
   return a0 < b0 + bbytes && b0 < a0 + abytes;
+}
+
+// one non-blocking side stream per device for the border strips (created on first use, never freed)
+constexpr int kSideDevices = 64;
+std::mutex g_side_mu;
+cudaStream_t g_side[kSideDevices] = {};
+
+cudaStream_t side_stream() {
+  int dev = 0;
+  if (cudaGetDevice(&dev) != cudaSuccess || dev < 0 || dev >= kSideDevices) return nullptr;
+  std::lock_guard<std::mutex> lk(g_side_mu);
+  if (!g_side[dev] && cudaStreamCreateWithFlags(&g_side[dev], cudaStreamNonBlocking) != cudaSuccess)
+    g_side[dev] = nullptr;
+  return g_side[dev];
 }
 
 int device_info(DevInfo *out) {
@@ -109,16 +125,20 @@ extern "C" int conv2d_single_pad(const float *in, int H, int W, const float *fil
   // One valid-mode launch of the per-K kernels: `src` (rows x cols, row pitch `pitch`) into `dst`
   // (output row pitch `po`). kBandNoSplit: the one-tile kernels everywhere in the padded call, so
   // interior and border outputs sum in the same order whatever the strip widths.
-  auto conv = [&](const float *src, int rows, int cols, long long pitch, float *dst, int po) -> int {
+  auto conv_on = [&](cudaStream_t st, int band_flag, const float *src, int rows, int cols, long long pitch,
+                     float *dst, int po) -> int {
     switch (K) {
 #define C2D_CALL_PAD(KK) \
-  case KK: return single_entry<KK>(src, rows, cols, f_use, dst, s, kBandNoSplit, dev, src, rows, pitch, po);
+  case KK: return single_entry<KK>(src, rows, cols, f_use, dst, st, band_flag, dev, src, rows, pitch, po);
       C2D_CALL_PAD(1) C2D_CALL_PAD(2) C2D_CALL_PAD(3) C2D_CALL_PAD(4) C2D_CALL_PAD(5) C2D_CALL_PAD(6)
       C2D_CALL_PAD(7) C2D_CALL_PAD(8) C2D_CALL_PAD(9) C2D_CALL_PAD(10) C2D_CALL_PAD(11) C2D_CALL_PAD(12)
       C2D_CALL_PAD(13) C2D_CALL_PAD(14) C2D_CALL_PAD(15)
 #undef C2D_CALL_PAD
       default: return CONV2D_EK;
     }
+  };
+  auto conv = [&](const float *src, int rows, int cols, long long pitch, float *dst, int po) -> int {
+    return conv_on(s, kBandNoSplit, src, rows, cols, pitch, dst, po);
   };
   if (!pad) {
     const int rc = conv(in, H, W, W, out, W - K + 1);
@@ -129,8 +149,8 @@ extern "C" int conv2d_single_pad(const float *in, int H, int W, const float *fil
   // [pt, pt+H-K+1) x [pl, pl+W-K+1) reads only the image itself: one launch straight on `in`, writing
   // into `out` with row pitch W -- no extra pass over the image. The four border strips (top pt rows,
   // bottom pb rows, left pl / right pr columns of the rows between) each read a thin slice of E, which
-  // k_pad_image materialises (16-byte pitch) in the scratch pool. Images smaller than the filter,
-  // and K >= 9: all of E at once.
+  // k_pad_image materialises (16-byte pitch) in the scratch pool. Images smaller than the filter:
+  // all of E at once.
   const int pt = (K - 1) / 2, pb = K - 1 - pt, pl = pt, pr = pb;
   struct Strip {
     int er0, ec0, rows, cols;  // slice of E
@@ -138,9 +158,13 @@ extern "C" int conv2d_single_pad(const float *in, int H, int W, const float *fil
   };
   Strip strips[5];
   int ns = 0;
-  // K >= 9 (FMA-bound): the strips -- latency-bound launches on images a few rows or columns wide --
-  // cost more than one extra pass over the image (8192^2 K=15: 0.70 vs 0.67 ms), so E is padded whole;
-  // K < 9 (HBM-bound): interior + strips (8192^2 K=3: 0.137 vs 0.197 ms). Same bits either way.
+  // The strips are latency-bound launches on images a few rows or columns wide: they run on a side
+  // stream, concurrently with the interior (forked after the scratch allocation, joined before the
+  // scratch is released), with the shared-memory filter so they never wait for the interior's use of
+  // the constant slot. Same one-tile kernels, same bits. K < 9 (HBM-bound): 8192^2 K=3 'same' 0.197 ms
+  // with the whole image padded -> 0.137 ms strips after the interior -> 0.128 ms concurrent strips.
+  // K >= 9 (FMA-bound): the FMA-saturating interior leaves the strips no room, so the whole image is
+  // padded instead (8192^2 K=15: 0.67 vs 0.68 ms).
   const bool interior = H >= K && W >= K && K < 9;
   const int WE = W + K - 1;  // width of E
   if (!interior) {
@@ -164,6 +188,15 @@ extern "C" int conv2d_single_pad(const float *in, int H, int W, const float *fil
     return CONV2D_EALLOC;
   }
   int rc = CONV2D_OK;
+  cudaStream_t ss = s;  // the strips' stream
+  cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
+  if (interior && ns > 0) {
+    cudaStream_t side = side_stream();
+    if (side && cudaEventCreateWithFlags(&ev_fork, cudaEventDisableTiming) == cudaSuccess &&
+        cudaEventCreateWithFlags(&ev_join, cudaEventDisableTiming) == cudaSuccess &&
+        cudaEventRecord(ev_fork, s) == cudaSuccess && cudaStreamWaitEvent(side, ev_fork, 0) == cudaSuccess)
+      ss = side;
+  }
   for (int t = 0; t < ns && rc == CONV2D_OK; ++t) {
     const Strip &st = strips[t];
     const long long p4 = (st.cols + 3) / 4 * 4;
@@ -172,12 +205,19 @@ extern "C" int conv2d_single_pad(const float *in, int H, int W, const float *fil
     long long blocks = (quads + 255) / 256;
     const long long cap = static_cast<long long>(dev.num_sms) * 8;
     if (blocks > cap) blocks = cap;
-    k_pad_image<<<static_cast<unsigned>(blocks), 256, 0, s>>>(in, H, W, buf, st.rows, st.cols, p4 / 4, pt, pl,
-                                                              pad == CONV2D_PAD_REPLICATE ? 1 : 0, st.er0, st.ec0);
+    k_pad_image<<<static_cast<unsigned>(blocks), 256, 0, ss>>>(in, H, W, buf, st.rows, st.cols, p4 / 4, pt, pl,
+                                                               pad == CONV2D_PAD_REPLICATE ? 1 : 0, st.er0, st.ec0);
     if (cudaGetLastError() != cudaSuccess) rc = CONV2D_ECUDA;
-    if (rc == CONV2D_OK) rc = conv(buf, st.rows, st.cols, p4, out + st.out_off, W);
+    if (rc == CONV2D_OK)
+      rc = conv_on(ss, ss == s ? kBandNoSplit : kBandSmemFilter, buf, st.rows, st.cols, p4, out + st.out_off, W);
   }
   if (rc == CONV2D_OK && interior) rc = conv(in, H, W, W, out + static_cast<long long>(pt) * W + pl, W);
+  if (ss != s) {  // join the strips back into the caller's stream (also on an error: nothing may dangle)
+    if (cudaEventRecord(ev_join, ss) != cudaSuccess || cudaStreamWaitEvent(s, ev_join, 0) != cudaSuccess)
+      rc = CONV2D_ECUDA;
+  }
+  if (ev_fork) cudaEventDestroy(ev_fork);
+  if (ev_join) cudaEventDestroy(ev_join);
   if (scratch) cudaFreeAsync(scratch, s);
   if (f_rot) cudaFreeAsync(f_rot, s);
   return rc;

@@ -225,7 +225,8 @@ int launch_single_default(const float *in, int H, int W, const float *filt, floa
   launch_single_v<K, UU, FS, PFF, G, HALO>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1, P, Po)
 #define C2D_SP(GG, UU, PFF, RR, CLL) \
   launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(in, H, W, filt, out, stream, band_h, dev, 1, in2, H1, P, Po)
-  const bool no_split = band_h == kBandNoSplit;  // internal callers that need the one-tile kernel's bits
+  const bool force_smem = band_h == kBandSmemFilter;
+  const bool no_split = band_h == kBandNoSplit || force_smem;  // internal callers: the one-tile kernel's bits
   if (no_split) band_h = 0;
   // Narrow images with large K (latency regime: a full wave of one-warp tiles leaves bands of a few
   // rows, and the K-1 prologue rows of Alg. 2 case 1 dominate): filter rows split over a cluster of 2
@@ -249,7 +250,7 @@ int launch_single_default(const float *in, int H, int W, const float *filt, floa
   // (tools/small_sizes2.py, back-to-back calls: 1024^2 K=3 12.1 -> 8.0 us, K=5 12.0 -> 10.3 us)
   const long long px = static_cast<long long>(H) * W;
   const bool small = px <= 512LL * 512 || (K <= 5 && px <= 1024LL * 1024);
-  if (!constant_ok || (K < 11 && small))
+  if (!constant_ok || force_smem || (K < 11 && small))
     return (K <= 7) ? C2D_LS(2, FSRC_SMEM, 1, 0) : C2D_LS(1, FSRC_SMEM, 1, 0);
   if constexpr (K <= 5) {
     if (K <= 3 && W > 1024) return C2D_LS(2, FSRC_CONST, 1, 0);
