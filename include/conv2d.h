@@ -23,15 +23,19 @@
  *     per-K slot of the module's __constant__ bank; an event recorded behind each kernel orders the
  *     next overwrite of the slot, so concurrent calls on different streams never see each other's
  *     filter (same-K calls on different streams are serialised by that wait). Under CUDA-graph
- *     capture the filter is staged per CTA in shared memory instead. Multi-channel filters are
- *     staged per CTA in shared memory.
+ *     capture, and for small images (<= 512^2, or <= 1024^2 with K <= 5, where the staging copy
+ *     would cost more than it saves), the filter is staged per CTA in shared memory instead.
+ *     Multi-channel filters are staged per CTA in shared memory.
  *   - Return value: 0 when the work was enqueued. A negative CONV2D_E* code when an argument is
  *     invalid (nothing was launched) or the launch itself failed. Asynchronous execution errors
  *     surface at the caller's next synchronisation, as in CUDA.
  *   - Stride 1, no padding ("valid"): Ho = H-K+1, Wo = W-K+1. Square K x K filters, 1 <= K <= 15
  *     (R14). Every output element is written exactly once and never read.
  *   - Arithmetic: fp32 FMA, accumulated per output in filter-row / filter-column order (multi:
- *     filter-row, channel, filter-column). Acceptance vs the CPU oracle: |gpu - ref| <= 1e-5 *
+ *     filter-row, channel, filter-column). Exception: single-channel images with W <= 1024 and
+ *     K >= 11 (when not captured into a graph) run the filter-row split kernel, which sums two
+ *     partial results (filter rows [0, K/2) and [K/2, K)) -- same tolerance, not the same bits as the
+ *     one-pass order. Results never depend on the band height or the row-band split. Acceptance vs the CPU oracle: |gpu - ref| <= 1e-5 *
  *     sum|x||w| per element (BASELINE.json north_star). No fast-math, denormals preserved.
  */
 #ifndef CONV2D_B200_H
