@@ -266,6 +266,9 @@ int launch_single_default(const float *in, int H, int W, const float *filt, floa
   } else if constexpr (K <= 11) {
     return C2D_LS(1, FSRC_CONST, 4, 2);
   } else {
+    // K = 12-14, wide: the cp.async ring with the guarded prologue (variant 15: 8192^2 K=13 155 -> 161
+    // Gpx/s, 4096^2 128 -> 132); K = 15 measured equal either way and keeps the register row fetch
+    if (K <= 14 && W >= 4096) return C2D_LS(1, FSRC_CONST, 4, 1);
     if (W >= 4096) return C2D_LS(1, FSRC_CONST, 1, 1);
     return C2D_LS(1, FSRC_CONST, 1, 2);
   }
@@ -299,6 +302,7 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
     case 8: if (constant_ok) return C2D_LS(2, FSRC_CONST, 8, 0); break;
     case 9: if (constant_ok) return C2D_LS(1, FSRC_CONST, 4, 2); break;
     case 13: if constexpr (K >= 5 && K <= 9) { if (constant_ok) return C2D_LS(2, FSRC_CONST, 4, 2); } break;
+    case 15: if constexpr (K >= 10) { if (constant_ok) return C2D_LS(1, FSRC_CONST, 4, 1); } break;
     default: break;
   }
   // filter-row split (conv2d_split.cuh; variants 10-12)

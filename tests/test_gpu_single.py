@@ -168,7 +168,7 @@ def test_config4_32768_k15_sampled(cuda_device):
         assert torch.equal(part, y[lo:hi])
 
 
-@pytest.mark.parametrize("variant", [1, 2, 3, 4, 5, 6, 7, 9, 13])
+@pytest.mark.parametrize("variant", [1, 2, 3, 4, 5, 6, 7, 9, 13, 15])
 def test_every_kernel_variant_bitwise_equal(cuda_device, variant):
     """Every instantiation (filter in shared / constant memory, 1 or 2 column chunks, guarded or
     unguarded band prologue/epilogue) of the one-warp-tile kernel gives the same bits as variant 1,
@@ -177,8 +177,8 @@ def test_every_kernel_variant_bitwise_equal(cuda_device, variant):
     shapes = [(40, 300), (77, 1030), (300, 517)]
     try:
         for K in (1, 2, 3, 5, 8, 9, 12, 15):
-            if variant == 13 and not 5 <= K <= 9:
-                continue  # variant 13 is instantiated for K = 5..9 only (elsewhere it means the default)
+            if (variant == 13 and not 5 <= K <= 9) or (variant == 15 and K < 10):
+                continue  # variants 13 / 15 are instantiated for K = 5..9 / K >= 10 only
             f = _filt(K, "rand", seed=K)
             for (dh, W) in shapes:
                 x = dev_image((K + dh, W), "img", seed=K * 7 + W)
