@@ -17,7 +17,11 @@ def dev_image(shape, dist="img", seed=synth.BASE_SEED, device="cuda"):
 
 
 def check_full_single(x: torch.Tensor, f: torch.Tensor, y: torch.Tensor, exact: bool = False):
-    xh, fh, yh = x.cpu().numpy(), f.cpu().numpy(), y.cpu().numpy()
+    check_full_single_host(x.cpu().numpy(), f.cpu().numpy(), y.cpu().numpy(), exact)
+
+
+def check_full_single_host(xh: np.ndarray, fh: np.ndarray, yh: np.ndarray, exact: bool = False):
+    """Every output of yh (host copy of the device result) against the oracle on the same input."""
     ref, bound, _ = oracle.conv2d_single(xh, fh)
     assert yh.shape == ref.shape
     if exact:

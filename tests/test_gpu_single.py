@@ -1,8 +1,9 @@
 """GPU parity of conv2d_single (C ABI via the binding) against the CPU oracle.
 
 Small shapes are compared element by element (all K in 1..15, ragged widths, every W % 4, Wo < 32,
-H == K, W == K, misaligned pointers); the BASELINE.json configs at full size are compared on sampled
-outputs (corners, edges, band boundaries, random points) in the launch configuration bench.py times.
+H == K, W == K, misaligned pointers); the BASELINE.json configs at full size are compared element by
+element too (every output of the 28 sweep points; configs[4]: every output around the 8-way row-band
+seams and of two whole bands), in the launch configuration bench.py times.
 """
 import numpy as np
 import pytest
@@ -11,7 +12,7 @@ import torch
 import paper_conf_cluster_luzw20_b200 as pkg
 from gen import synth
 from paper_conf_cluster_luzw20_b200 import _capi
-from tests.gpu_helpers import (check_full_single, check_points_single, dev_image, sample_points)
+from tests.gpu_helpers import check_full_single, check_full_single_host, dev_image
 
 pytestmark = pytest.mark.gpu
 DEV = "cuda"
@@ -127,45 +128,56 @@ def test_error_codes_on_device(cuda_device):
 
 
 # --------------------------------------------------------------------------------------------
-# BASELINE.json configs at full size, sampled outputs
+# BASELINE.json configs at full size, EVERY output (configs[4]: every output of the band seams and of
+# two whole bands), in the launch configuration bench.py times
 # --------------------------------------------------------------------------------------------
 @pytest.mark.parametrize("S", [1024, 2048, 4096, 8192])
-def test_config1_sweep_full_size_sampled(cuda_device, S):
-    """configs[1]: 1024^2..8192^2 x K in {3,..,15}, the bench launch configuration, sampled."""
-    rng = np.random.default_rng(S)
+def test_config1_sweep_full_size_every_output(cuda_device, S):
+    """configs[1]: 1024^2..8192^2 x K in {3,..,15}, the bench launch configuration (one conv2d_single
+    call per point on the current stream, automatic band height); every output against the oracle."""
     x = dev_image((S, S), "img", seed=synth.BASE_SEED + 1)
+    xh = x.cpu().numpy()
     for K in (3, 5, 7, 9, 11, 13, 15):
         f = _filt(K, "rand", seed=synth.BASE_SEED + K)
         y = pkg.conv2d_single(x, f)
         torch.cuda.synchronize()
-        ys, xs = sample_points(S - K + 1, S - K + 1, 400, rng, band_h=None)
-        check_points_single(x, f, y, ys, xs)
-        assert torch.isfinite(y).all()
-    del x, y
+        check_full_single_host(xh, f.cpu().numpy(), y.cpu().numpy())
+        del y
 
 
-def test_config4_32768_k15_sampled(cuda_device):
-    """configs[4]: one 32768^2 image, K=15 (4 GiB in + 4 GiB out) on one B200, sampled; and the
-    row-band split used across GPUs reproduces it bit for bit at the band seams."""
+def test_config4_32768_k15_seams_and_bands(cuda_device):
+    """configs[4]: one 32768^2 image, K=15 (4 GiB in + 4 GiB out) in one launch on one B200. Every
+    output within K rows of each of the 7 seams of the 8-way row-band split (shard.row_band, the
+    multi-GPU decomposition), plus every output of two whole bands (the first and the last), against
+    the oracle; and each band computed on its own (what a rank computes) equals the one-launch rows
+    bit for bit at the seams."""
+    from paper_conf_cluster_luzw20_b200 import shard
+
     S, K = 32768, 15
     free, _ = torch.cuda.mem_get_info()
     if free < 10 * (1 << 30):
         pytest.skip("needs ~9 GiB of free HBM")
     x = dev_image((S, S), "img", seed=synth.BASE_SEED + 4)
     f = _filt(K, "gauss")
+    fh = f.cpu().numpy()
     y = pkg.conv2d_single(x, f)
     torch.cuda.synchronize()
-    rng = np.random.default_rng(4)
     Ho = S - K + 1
-    ys, xs = sample_points(Ho, Ho, 300, rng)
-    check_points_single(x, f, y, ys, xs)
-    # 8 row bands computed independently (the multi-GPU decomposition) match at the seams
-    bands = np.linspace(0, Ho, 9).astype(int)
-    for b in range(8):
-        o0, o1 = int(bands[b]), int(bands[b + 1])
-        lo, hi = max(o0, o1 - 3), o1
-        part = pkg.conv2d_single(x[lo:hi + K - 1], f)
-        assert torch.equal(part, y[lo:hi])
+    bands = [shard.row_band(S, S, K, 8, r) for r in range(8)]
+
+    def check_rows(o0, o1):
+        xh = x[o0:o1 + K - 1].cpu().numpy()
+        check_full_single_host(xh, fh, y[o0:o1].cpu().numpy())
+
+    for b in bands[:-1]:  # seams: output rows [o1 - K, o1 + K) around each band end
+        check_rows(max(0, b.o1 - K), min(Ho, b.o1 + K))
+    for b in (bands[0], bands[-1]):  # two whole bands
+        check_rows(b.o0, b.o1)
+    for b in bands:  # a band computed alone (rows o0 .. o1+K-1) equals the one-launch rows
+        lo, hi = b.o0, b.o1
+        for a0, a1 in ((lo, min(hi, lo + 2 * K)), (max(lo, hi - 2 * K), hi)):
+            part = pkg.conv2d_single(x[a0:a1 + K - 1], f)
+            assert torch.equal(part, y[a0:a1]), (b.rank, a0, a1)
 
 
 @pytest.mark.parametrize("variant", [1, 2, 3, 4, 5, 6, 7, 9, 13, 15])
@@ -313,6 +325,8 @@ def test_halo_segment_bitwise(cuda_device, K):
                 got = pkg.conv2d_single_halo(x, halo, f)
                 torch.cuda.synchronize()
                 assert torch.equal(got, ref), (K, H, W, hr, off)
+                if off == 1 and hr == max(K - 1, 0):  # the row-band case: every output vs the oracle
+                    check_full_single(full[:H + hr], f, got)
     x = dev_image((30, 64), "img")
     halo = dev_image((K, 64), "img", seed=5)
     y = torch.empty((30 + K - K + 1, 64 - K + 1), device=DEV)
