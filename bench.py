@@ -2,18 +2,24 @@
 """Benchmark of the hot path (driver contract).
 
     python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference] [--workload NAME]
+                    [--batch B]
 
 Default workload = BASELINE.json configs[1], the workload its metric is quoted on: the single-channel
-sweep of 1024^2, 2048^2, 4096^2, 8192^2 fp32 images x K in {3,5,7,9,11,13,15} (28 convolutions).
-One "step" = one pass of the whole hot path over that sweep: every (size, K) point is one
-conv2d_single call on its own input/output buffers (so no point reads another's data from L2),
-largest images first. `value` = output pixels of all points of all ranks / time (Gpixel/s), timed on
-the device with CUDA events, L2 flushed (a 512 MiB write, then a 256 MiB read that evicts its dirty lines) between steps outside the timed region.
+sweep of 1024^2, 2048^2, 4096^2, 8192^2 fp32 images x K in {3,5,7,9,11,13,15} (28 points). Each
+point is a batch of B images (--batch, default 8) filtered with one filter: one conv2d_single_batch
+call per point (conv2d_single when a rank holds one image), on its own input/output buffers, largest
+images first. One "step" = one pass over all 28 points. `value` = output pixels of the whole job
+/ time (Gpixel/s), timed on the device with CUDA events, max over ranks, L2 flushed (a 512 MiB write,
+then a 256 MiB read that evicts its dirty lines) between steps outside the timed region.
 
-N > 1 (torchrun): every rank runs the same sweep on its own images (seeded by rank): weak scaling,
+Multi-GPU (--gpus N): one process per GPU over NCCL. Without torchrun's environment, bench.py
+re-launches itself under `python -m torch.distributed.run --nproc-per-node N` (fails loudly when
+fewer than N GPUs are visible). The batch of every point is split across ranks (shard.batch_range:
+rank p takes images [p*B/N, (p+1)*B/N)) -- a fixed total amount of work, so "scaling": "strong", and
 no data-path collective (north_star: "partitioned ... by image/batch ... no collective needed").
-Other workloads (--workload): config0, config2, config3 (GFLOP/s), config4 (32768^2 K=15; at N>1
-row bands with the NCCL halo exchange of shard.py).
+configs[2] / configs[3] (--workload config2 / config3) shard their N=32 / N=128 batches the same way;
+configs[4] (--workload config4, one 32768^2 image, K=15) is split into row bands with the (K-1)-row
+NCCL halo exchange of shard.py.
 
 --impl reference: the CPU oracle (this tier's reference arm) timed as it stands on the host cores,
 on a bounded sample of the same workload (rank 0 only).
@@ -68,40 +74,64 @@ def fp32_fma_peak_tflops(sm_mhz):
 class Point:
     """One conv call of a step: shapes, device buffers, algorithmic work."""
 
-    def __init__(self, kind, name, dims, K, padding="valid", flip=False, halo_rows=0):
+    def __init__(self, kind, name, dims, K, padding="valid", flip=False, halo_rows=0, batch=1):
         self.kind, self.name, self.dims, self.K = kind, name, dims, K
         self.padding, self.flip, self.halo_rows = padding, flip, halo_rows  # N4 / N3 variants (single)
+        self.batch = batch  # single: images per point (the whole job's batch); multi: dims[0]
+        self.n0 = 0         # this rank's images [n0, n0 + n_local) of the batch (shard.batch_range)
+        self.n_local = self.images
         self.x = self.f = self.y = self.halo = None
 
     @property
-    def out_px(self):
+    def images(self):
+        return self.batch if self.kind == "single" else self.dims[0]
+
+    @property
+    def out_px_image(self):
+        """output elements of one image (single: pixels; multi: F output planes)"""
         if self.kind == "single":
             H, W = self.dims
             if self.padding != "valid":
                 return H * W
             return (H - self.K + 1) * (W - self.K + 1)
         N, C, H, W, F = self.dims
-        return N * F * (H - self.K + 1) * (W - self.K + 1)
+        return F * (H - self.K + 1) * (W - self.K + 1)
+
+    @property
+    def out_px(self):
+        """output elements of the whole point (all images of the batch)"""
+        return self.out_px_image * self.images
 
     @property
     def flops(self):
         C = 1 if self.kind == "single" else self.dims[1]
         return 2.0 * self.out_px * C * self.K * self.K
 
+    def local_units(self, unit):
+        """units this rank computes per step"""
+        per_img = self.out_px_image if unit == "Gpixel/s" else self.flops / self.images
+        return per_img * self.n_local
+
     @property
     def bytes(self):
-        """compulsory HBM bytes: inputs + outputs + filters"""
+        """compulsory HBM bytes of the whole point: inputs + outputs + filters"""
         if self.kind == "single":
             H, W = self.dims
-            return 4.0 * (H * W + self.out_px + self.K * self.K)
+            return 4.0 * (self.batch * H * W + self.out_px + self.K * self.K)
         N, C, H, W, F = self.dims
         return 4.0 * (N * C * H * W + self.out_px + F * C * self.K * self.K)
 
     def in_bytes(self):
+        """input bytes of this rank's images"""
         if self.kind == "single":
-            return 4 * self.dims[0] * self.dims[1]
+            return 4 * self.n_local * self.dims[0] * self.dims[1]
         N, C, H, W, F = self.dims
-        return 4 * N * C * H * W
+        return 4 * self.n_local * C * H * W
+
+    def local_bound_seconds(self, peaks, sm_mhz):
+        """roofline time of this rank's share of the point"""
+        _, t = self.bound(peaks, sm_mhz)
+        return t * self.n_local / max(1, self.images)
 
     def filt_bytes(self):
         C = 1 if self.kind == "single" else self.dims[1]
@@ -114,12 +144,18 @@ class Point:
         return ("hbm", t_mem) if t_mem >= t_fma else ("alu", t_fma)
 
 
-def workload_points(name):
+DEFAULT_SWEEP_BATCH = 8
+
+
+def workload_points(name, batch=None):
+    """The points of one step of a workload. batch: images per single-channel point (sweep default
+    DEFAULT_SWEEP_BATCH, config0 default 1)."""
     if name == "sweep":
-        return [Point("single", f"{S}^2 K={K}", (S, S), K) for S in SWEEP_SIZES for K in SWEEP_KS], \
+        b = DEFAULT_SWEEP_BATCH if batch is None else batch
+        return [Point("single", f"{S}^2 K={K}", (S, S), K, batch=b) for S in SWEEP_SIZES for K in SWEEP_KS], \
             "Gpixel/s"
     if name == "config0":
-        return [Point("single", "256^2 K=3", (256, 256), 3)], "Gpixel/s"
+        return [Point("single", "256^2 K=3", (256, 256), 3, batch=batch or 1)], "Gpixel/s"
     if name == "config2":
         return [Point("multi", "N32 C64 F64 56^2 K3", (32, 64, 56, 56, 64), 3)], "GFLOP/s"
     if name == "config3":
@@ -138,6 +174,22 @@ def workload_points(name):
     raise SystemExit(f"unknown workload {name}")
 
 
+def shard_points(points, world, rank):
+    """Split every point's batch across ranks (shard.batch_range): rank p computes images
+    [n0, n0 + n_local). No data-path collective; the union over ranks is the whole job."""
+    from paper_conf_cluster_luzw20_b200.shard import batch_range
+
+    for p in points:
+        n0, n1 = batch_range(p.images, world, rank)
+        p.n0, p.n_local = n0, n1 - n0
+    return points
+
+
+def job_units(points, unit):
+    """units of the whole job per step (all ranks)"""
+    return sum(p.out_px if unit == "Gpixel/s" else p.flops for p in points)
+
+
 # PAPER.md Table I (P:335-352): name, IH = IW, FN, FH = FW
 TABLE1 = [("CONV1", 28, 128, 3), ("CONV2", 56, 64, 3), ("CONV3", 12, 64, 5), ("CONV4", 14, 16, 5),
           ("CONV5", 24, 256, 5), ("CONV6", 24, 64, 5), ("CONV7", 28, 16, 5), ("CONV8", 28, 512, 3),
@@ -145,10 +197,11 @@ TABLE1 = [("CONV1", 28, 128, 3), ("CONV2", 56, 64, 3), ("CONV3", 12, 64, 5), ("C
 
 WORKLOAD_DESC = {
     "sweep": "BASELINE.json configs[1]: single-channel sweep, 1024^2/2048^2/4096^2/8192^2 x K in "
-             "{3,5,7,9,11,13,15} (28 conv2d_single calls per step, largest first)",
-    "config0": "BASELINE.json configs[0]: 256x256, K=3",
-    "config2": "BASELINE.json configs[2]: N=32, C=F=64, 56x56, K=3",
-    "config3": "BASELINE.json configs[3]: N=128, C=3, F=64, 224x224, K=7",
+             "{3,5,7,9,11,13,15}, a batch of B images per point (28 conv2d_single_batch calls per step, "
+             "largest first; the batch split across ranks)",
+    "config0": "BASELINE.json configs[0]: 256x256, K=3 (batch B, default 1)",
+    "config2": "BASELINE.json configs[2]: N=32, C=F=64, 56x56, K=3 (batch split across ranks)",
+    "config3": "BASELINE.json configs[3]: N=128, C=3, F=64, 224x224, K=7 (batch split across ranks)",
     "config4": "BASELINE.json configs[4]: 32768x32768, K=15 (row bands + NCCL halo at N>1)",
     "table1": "PAPER.md Table I (P:335-352): 11 layers x C in {1,3}, N=128 (22 conv2d_multi calls per step)",
     "pad": "SURVEY 8(f) N4: 8192^2, K in {3,15}, 'same' zero padding / 'same' replicate padding + true "
@@ -158,29 +211,34 @@ WORKLOAD_DESC = {
 }
 
 
-def materialise(points, rank, world, device):
+def materialise(points, device):
+    """Device buffers of this rank's images of every point, generated in place from the global
+    element index (gen/synth.py): the shards of all ranks together are the one-GPU batch, bit for bit."""
     import torch
 
     from gen import synth
 
     for i, p in enumerate(points):
-        seed = synth.BASE_SEED + 1000 * rank + i
+        seed = synth.BASE_SEED + i
+        if p.n_local == 0:
+            continue
         if p.kind == "single":
             H, W = p.dims
-            full = synth.fill_torch(seed, synth.TAG_INPUT, (H, W), "img", device=device)
+            full = synth.fill_torch(seed, synth.TAG_INPUT, (p.n_local, H, W), "img", start=p.n0 * H * W,
+                                    device=device)
             hr = p.halo_rows
-            p.x = full[:H - hr].clone() if hr else full
-            p.halo = full[H - hr:].clone() if hr else None
+            p.x = full[:, :H - hr].contiguous() if hr else full
+            p.halo = full[:, H - hr:].contiguous() if hr else None
             del full
             p.f = torch.from_numpy(synth.make_filter(seed, p.K, "rand")[0, 0]).to(device)
-            p.y = (torch.empty((H, W), device=device) if p.padding != "valid" else
-                   torch.empty((H - p.K + 1, W - p.K + 1), device=device))
+            Ho, Wo = (H, W) if p.padding != "valid" else (H - p.K + 1, W - p.K + 1)
+            p.y = torch.empty((p.n_local, Ho, Wo), device=device)
         else:
             N, C, H, W, F = p.dims
-            p.x = synth.fill_torch(seed, synth.TAG_INPUT, (N, C, H, W), "img" if C < 8 else "sym",
-                                   device=device)
+            p.x = synth.fill_torch(seed, synth.TAG_INPUT, (p.n_local, C, H, W), "img" if C < 8 else "sym",
+                                   start=p.n0 * C * H * W, device=device)
             p.f = torch.from_numpy(synth.make_filter(seed, p.K, "he", F=F, C=C)).to(device)
-            p.y = torch.empty((N, F, H - p.K + 1, W - p.K + 1), device=device)
+            p.y = torch.empty((p.n_local, F, H - p.K + 1, W - p.K + 1), device=device)
 
 
 # ------------------------------------------------------------------------------------------------
@@ -252,16 +310,20 @@ def run_ours(args):
     world = int(os.environ.get("WORLD_SIZE", "1"))
     rank = int(os.environ.get("RANK", "0"))
     local = int(os.environ.get("LOCAL_RANK", "0"))
+    if world != args.gpus:
+        raise SystemExit(f"bench.py: --gpus {args.gpus} but WORLD_SIZE={world} (launch one rank per GPU)")
     if world > 1:
+        if torch.cuda.device_count() < world:
+            raise SystemExit(f"bench.py: {world} ranks but only {torch.cuda.device_count()} visible GPUs")
         torch.cuda.set_device(local)
         dist.init_process_group("nccl", device_id=torch.device("cuda", local))
     device = torch.device("cuda", local)
     torch.cuda.set_device(device)
     peaks = load_peaks()
 
-    points, unit = workload_points(args.workload)
+    points, unit = workload_points(args.workload, args.batch)
     if args.variant:
-        pkg._capi.debug_set_variant(args.variant)
+        pkg._capi.debug_set_variant(args.variant)  # tuning library (tools / A-B runs only)
     rowband = args.workload == "config4" and world > 1
     band = None
     if rowband:
@@ -281,11 +343,13 @@ def run_ours(args):
                                               start=band.o0 * W, device=device)
         p.f = torch.from_numpy(synth.make_filter(synth.BASE_SEED, p.K, "gauss")[0, 0]).to(device)
         p.y = torch.empty((band.out_rows, W - p.K + 1), device=device)
+        p.n0, p.n_local = 0, 1
         if args.halo in ("p2p", "ipc"):  # every neighbour's rows are written before any rank reads them
             torch.cuda.synchronize()
             dist.barrier()
     else:
-        materialise(points, rank, world, device)
+        shard_points(points, world, rank)
+        materialise(points, device)
     stream = torch.cuda.current_stream(device)
     flush = torch.empty(512 * (1 << 20) // 4, dtype=torch.float32, device=device)
     flush_rd = torch.ones(256 * (1 << 20) // 4, dtype=torch.float32, device=device)
@@ -298,6 +362,7 @@ def run_ours(args):
 
     use_graph = not rowband and (args.graph == "on" or (args.graph == "auto" and args.workload == "config0"))
     capturing = [False]
+    active = [i for i, p in enumerate(points) if p.n_local > 0]
 
     def run_point(p, on=None):
         st = None if capturing[0] else (on if on is not None else stream)  # capture: torch's capture stream
@@ -306,11 +371,13 @@ def run_ours(args):
         elif rowband:
             shard.rowband_conv2d_single(p.x, p.f, band, p.y)
         elif p.kind == "single" and p.halo is not None:
-            pkg.conv2d_single_halo(p.x, p.halo, p.f, out=p.y, stream=st)
+            pkg.conv2d_single_halo(p.x[0], p.halo[0], p.f, out=p.y[0], stream=st)
         elif p.kind == "single" and (p.padding != "valid" or p.flip):
-            pkg.conv2d_single_pad(p.x, p.f, p.padding, p.flip, out=p.y, stream=st)
+            pkg.conv2d_single_pad(p.x[0], p.f, p.padding, p.flip, out=p.y[0], stream=st)
+        elif p.kind == "single" and p.n_local == 1:
+            pkg.conv2d_single(p.x[0], p.f, out=p.y[0], stream=st)
         elif p.kind == "single":
-            pkg.conv2d_single(p.x, p.f, out=p.y, stream=st)
+            pkg.conv2d_single_batch(p.x, p.f, out=p.y, stream=st)
         elif args.multi_impl == "tc":
             pkg.conv2d_multi_tc(p.x, p.f, out=p.y, stream=st)
         else:
@@ -326,35 +393,35 @@ def run_ours(args):
     def in_px(p):
         return p.dims[0] * p.dims[1] if p.kind == "single" else p.dims[0] * p.dims[2] * p.dims[3]
 
-    px_max = max(in_px(p) for p in points)
+    px_max = max(in_px(points[i]) for i in active) if active else 0
     lanes = {}
     conc = args.concurrency if args.concurrency != "auto" else ("small" if args.workload == "table1" else "serial")
     if conc == "small" and not rowband and not use_graph:
-        for p in points:
-            if in_px(p) < px_max:
-                lanes.setdefault(p.K, torch.cuda.Stream(device))
+        for i in active:
+            if in_px(points[i]) < px_max:
+                lanes.setdefault(points[i].K, torch.cuda.Stream(device))
 
     def step(evs=None, dom=None, dom_evs=None):
         """one pass over the workload; evs: an event after every point (warm-up breakdown);
         dom/dom_evs: events bracketing the dominant point only (timed steps: 2 extra events)"""
         if lanes and evs is None:
-            big = [(i, p) for i, p in enumerate(points) if in_px(p) == px_max]
-            small = [(i, p) for i, p in enumerate(points) if in_px(p) < px_max]
-            for i, p in big:
+            big = [i for i in active if in_px(points[i]) == px_max]
+            small = [i for i in active if in_px(points[i]) < px_max]
+            for i in big:
                 if dom_evs is not None and i == dom:
                     dom_evs[0].record(stream)
-                run_point(p)
+                run_point(points[i])
                 if dom_evs is not None and i == dom:
                     dom_evs[1].record(stream)
             fork = torch.cuda.Event()
             fork.record(stream)
             for ln in lanes.values():
                 ln.wait_event(fork)
-            for i, p in small:
-                ln = lanes[p.K]
+            for i in small:
+                ln = lanes[points[i].K]
                 if dom_evs is not None and i == dom:
                     dom_evs[0].record(ln)
-                run_point(p, ln)
+                run_point(points[i], ln)
                 if dom_evs is not None and i == dom:
                     dom_evs[1].record(ln)
             for ln in lanes.values():
@@ -362,15 +429,17 @@ def run_ours(args):
                 j.record(ln)
                 stream.wait_event(j)
             return
-        for i, p in enumerate(points):
+        for i in range(n):
             if dom_evs is not None and i == dom:
                 dom_evs[0].record(stream)
-            run_point(p)
+            if i in active_set:
+                run_point(points[i])
             if dom_evs is not None and i == dom:
                 dom_evs[1].record(stream)
             if evs is not None:
                 evs[i + 1].record(stream)
 
+    active_set = set(active)
     # warm-up steps: per-point events give the per-point breakdown and pick the dominant kernel
     warm_ms = [0.0] * n
     counted = max(1, args.warmup - 1)  # the first warm-up step pays one-time setup: not counted
@@ -383,7 +452,7 @@ def run_ours(args):
         if w > 0 or args.warmup == 1:
             for i in range(n):
                 warm_ms[i] += evs[i].elapsed_time(evs[i + 1]) / counted
-    dom = max(range(n), key=lambda i: warm_ms[i])
+    dom = max(range(n), key=lambda i: warm_ms[i] if i in active_set else -1.0)
     if lanes:  # one untimed step in the timed steps' (concurrent) form
         l2_flush()
         step()
@@ -404,8 +473,12 @@ def run_ours(args):
         graph.replay()
         torch.cuda.synchronize()
 
-    # timed steps: events at the step boundaries and around the dominant kernel only
+    # timed steps: barrier + synchronize on both sides; events at the step boundaries and around the
+    # dominant kernel only
     step_events = [[torch.cuda.Event(enable_timing=True) for _ in range(4)] for _ in range(args.steps)]
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
     with ClockSampler(local) as clk:
         for s in range(args.steps):
             l2_flush()  # L2 flush, outside [ev0, ev3]
@@ -426,39 +499,46 @@ def run_ours(args):
     total_ms = sum(ev[0].elapsed_time(ev[3]) for ev in step_events)
     dom_ms = sum(ev[1].elapsed_time(ev[2]) for ev in step_events) / args.steps
     per_point_ms = list(warm_ms)
-    if world > 1:
+    launches_local = sum(1 for _ in active) * args.steps * (2 if rowband and args.halo == "nccl" and not band.is_last
+                                                            else 1)
+    if world > 1:  # max over ranks of the timed region; sum of the kernel launches
         t = torch.tensor([total_ms], dtype=torch.float64, device=device)
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
         total_ms = float(t.item())
-
-    units_per_step_rank = sum(p.out_px if unit == "Gpixel/s" else p.flops for p in points)
-    if rowband:
-        units_per_step = sum(p.out_px for p in points)  # the one image, split over ranks
+        c = torch.tensor([launches_local], dtype=torch.int64, device=device)
+        dist.all_reduce(c, op=dist.ReduceOp.SUM)
+        launches = int(c.item())
     else:
-        units_per_step = units_per_step_rank * world
+        launches = launches_local
+
+    units_per_step = job_units(points, unit)  # the whole job: every rank's share (row bands: the one image)
     value = units_per_step * args.steps / (total_ms * 1e-3) / 1e9
 
     clocks = clk.summary()
     sm_mhz_peak = peaks["sm_max_mhz"]
 
-    # roofline of the dominant kernel (largest share of the step), timed inside the timed steps
+    # roofline of the dominant kernel (largest share of this rank's step), timed inside the timed steps:
+    # this rank's share of the point (its images, or its row band)
     dp = points[dom]
     dkind, _ = dp.bound(peaks, sm_mhz_peak)
     dsec = dom_ms * 1e-3
+    share = (band.out_rows / (dp.dims[0] - dp.K + 1)) if rowband else dp.n_local / max(1, dp.images)
+    d_flops, d_bytes = dp.flops * share, dp.bytes * share
     if dp.kind == "multi" and args.multi_impl == "tc":
         # tensor-core variant: the executed TF32 MMA flops (3 per useful product, the 3xTF32 split)
         # against the tf32 tensor peak (measured bf16 burst x the nominal tf32/bf16 ratio)
-        roof = {"bound": "tensor", "achieved": 3 * dp.flops / dsec / 1e12,
+        roof = {"bound": "tensor", "achieved": 3 * d_flops / dsec / 1e12,
                 "peak": peaks["bf16_tflops"] * TF32_PER_BF16, "unit": "TFLOP/s",
                 "note": "executed tf32 MMA TFLOP/s = 3 x useful (3xTF32); peak = bf16 burst x 1.1/2.25"}
     elif dkind == "hbm":
-        roof = {"bound": "hbm", "achieved": dp.bytes / dsec / 1e9, "peak": peaks["hbm_gbs"], "unit": "GB/s"}
+        roof = {"bound": "hbm", "achieved": d_bytes / dsec / 1e9, "peak": peaks["hbm_gbs"], "unit": "GB/s"}
     else:
-        roof = {"bound": "alu", "achieved": dp.flops / dsec / 1e12, "peak": fp32_fma_peak_tflops(sm_mhz_peak),
+        roof = {"bound": "alu", "achieved": d_flops / dsec / 1e12, "peak": fp32_fma_peak_tflops(sm_mhz_peak),
                 "unit": "TFLOP/s"}
     roof["frac"] = roof["achieved"] / roof["peak"]
     roof["kernel"] = (f"conv2d_multi_tc {dp.name}" if dp.kind == "multi" and args.multi_impl == "tc"
-                      else f"conv2d_{dp.kind} {dp.name}")
+                      else f"conv2d_{dp.kind} {dp.name}" + (f" x{dp.n_local} images" if dp.kind == "single"
+                                                            and dp.n_local > 1 else ""))
     roof["share_of_step"] = dom_ms / max(total_ms / args.steps, 1e-12)
     roof["launch_ms"] = round(dom_ms, 5)
     roof["peak_source"] = (peaks["source"] if dkind == "hbm" or roof["bound"] == "tensor" else
@@ -468,13 +548,19 @@ def run_ours(args):
 
     sweep = []
     for i, p in enumerate(points):
-        kind, t_roof = p.bound(peaks, sm_mhz_peak)
+        if i not in active_set:
+            continue
+        kind, _ = p.bound(peaks, sm_mhz_peak)
         t = per_point_ms[i] * 1e-3
-        sweep.append({"point": p.name, "ms": round(per_point_ms[i], 5),
-                      ("gpx_s" if unit == "Gpixel/s" else "gflop_s"):
-                          round((p.out_px if unit == "Gpixel/s" else p.flops) / t / 1e9, 2),
+        t_roof = (p.local_bound_seconds(peaks, sm_mhz_peak) if not rowband else
+                  p.bound(peaks, sm_mhz_peak)[1] * share)
+        u = (p.local_units(unit) if not rowband else p.out_px * share)
+        sweep.append({"point": p.name, "images": p.n_local, "ms": round(per_point_ms[i], 5),
+                      ("gpx_s" if unit == "Gpixel/s" else "gflop_s"): round(u / t / 1e9, 2),
                       "bound": kind, "roofline_frac": round(t_roof / t, 4)})
+    t_roof_step = sum(points[i].local_bound_seconds(peaks, sm_mhz_peak) for i in active) if not rowband else None
 
+    batched = points[0].kind == "single" and not rowband and args.workload in ("sweep", "config0")
     line = {
         "metric": BASELINE_METRIC,
         "metric_detail": f"{unit} of the {args.workload} workload (whole job, all ranks)",
@@ -485,49 +571,58 @@ def run_ours(args):
         "warmup": args.warmup,
         "ms_per_step": round(total_ms / args.steps, 5),
         "higher_is_better": True,
-        "scaling": "strong" if rowband else "weak",
+        "scaling": "strong" if (world > 1 or rowband or args.workload in ("sweep", "config2", "config3", "config0"))
+        else "weak",
         "vs_baseline": None,
         "dtype": "f32",
         "data": "synthetic (seeded counter-based generator, gen/synth.py)",
         "config": {"workload": WORKLOAD_DESC[args.workload],
+                   **({"batch": points[0].batch} if batched else {}),
                    **({"multi_impl": args.multi_impl} if points[0].kind == "multi" else {}),
                    "l2": "512 MiB write + 256 MiB read between timed steps (outside the events) + distinct buffers per "
-                         "conv; 8192^2 inputs also exceed L2",
+                         "point; 8192^2 inputs also exceed L2",
                    "parallelism": (("row bands + NCCL halo" if args.halo == "nccl" else
                                     f"row bands, halo read in place from the neighbour ({args.halo}, NVLink)")
                                    if rowband else
-                                   ("replicas (independent images per rank)" if world > 1 else "1 GPU")),
-                   "filter": "rand (2u-1)/K", "input": "img u in [0,1)"},
+                                   (f"batch split over {world} ranks (shard.batch_range), no collective"
+                                    if world > 1 else "1 GPU")),
+                   "filter": "rand (2u-1)/K" if points[0].kind == "single" else "he",
+                   "input": "img u in [0,1)"},
         "roofline": roof,
-        "gpu_launches": n * args.steps * (2 if rowband and args.halo == "nccl" and not band.is_last else 1),
+        "roofline_step_frac": (round(t_roof_step / (total_ms / args.steps * 1e-3), 4) if t_roof_step else None),
+        "gpu_launches": launches,
         "clocks": clocks,
         "points_warmup": sweep,
-        "points_note": "per-point times from the warm-up steps (an event after every call); the timed "
+        "points_note": "per-point times (this rank) from the warm-up steps (an event after every call); the timed "
                        "steps carry events only at the step boundaries and around the dominant kernel",
     }
     if lanes:
-        line["config"]["concurrency"] = (f"the {sum(in_px(p) == px_max for p in points)} largest calls serially on "
-                                         f"one stream, the other {sum(in_px(p) < px_max for p in points)} on "
-                                         f"{len(lanes)} streams (one per K), joined every step")
+        line["config"]["concurrency"] = (f"the {sum(in_px(points[i]) == px_max for i in active)} largest calls "
+                                         f"serially on one stream, the others on {len(lanes)} streams (one per K), "
+                                         f"joined every step")
     if graph is not None:
         line["config"]["timing"] = ("CUDA graph of the step (captured once, replayed per timed step): "
                                     "device time without per-call host overhead")
 
     # end to end through the public API with host buffers (pinned), copies inside the timed region
     if not rowband and not args.no_e2e:
-        e2e = run_e2e(points, unit, args, device)
+        e2e = run_e2e([points[i] for i in active], unit, args, device)
         if world > 1:  # whole job: every rank moved its own images; time = max over ranks
-            t = torch.tensor([e2e["ms_per_step"]], dtype=torch.float64, device=device)
-            dist.all_reduce(t, op=dist.ReduceOp.MAX)
-            ms = float(t.item())
-            e2e["value"] = round(e2e["value"] * e2e["ms_per_step"] / ms * world, 3)
+            t = torch.tensor([e2e["ms_per_step"], e2e["h2d_bytes_per_step"], e2e["d2h_bytes_per_step"]],
+                             dtype=torch.float64, device=device)
+            tm = t[:1].clone()
+            dist.all_reduce(tm, op=dist.ReduceOp.MAX)
+            tb = t[1:].clone()
+            dist.all_reduce(tb, op=dist.ReduceOp.SUM)
+            ms = float(tm.item())
+            e2e["value"] = round(units_per_step * e2e["steps"] / (ms * e2e["steps"] * 1e-3) / 1e9, 3)
             e2e["ms_per_step"] = round(ms, 3)
-            e2e["h2d_bytes_per_step"] *= world
-            e2e["d2h_bytes_per_step"] *= world
+            e2e["h2d_bytes_per_step"] = int(tb[0].item())
+            e2e["d2h_bytes_per_step"] = int(tb[1].item())
         line["e2e"] = e2e
 
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
-        line["cpu_baseline"] = cpu_baseline(args.workload, budget_s=args.cpu_budget)
+        line["cpu_baseline"] = cpu_baseline(args.workload, budget_s=args.cpu_budget, batch=args.batch)
 
     if world > 1:
         dist.barrier()
@@ -538,14 +633,10 @@ def run_ours(args):
 
 def run_e2e(points, unit, args, device):
     """Same metric through the user-facing host-buffer call (C ABI conv2d_single_host: chunked
-    H2D / kernel / D2H pipeline; multi-channel: torch copies around conv2d_multi), pinned host
-    tensors, every byte of every input copied in and every output copied out inside the events.
-    Consecutive calls alternate between two streams (independent images), as a user pipelining a
-    batch of images would, so one call's device->host copies overlap the next call's host->device."""
-    import torch
-
-    import paper_conf_cluster_luzw20_b200 as pkg
-
+    H2D / kernel / D2H pipeline, one call per image; multi-channel: torch copies around conv2d_multi),
+    pinned host tensors, every byte of every input copied in and every output copied out inside the
+    events. Consecutive calls alternate between two streams (independent images), as a user pipelining
+    a batch of images would, so one call's device->host copies overlap the next call's host->device."""
     # Keep the host side on the GPU's NUMA node: the pinned staging buffers are first-touched by
     # this thread, so they land in memory local to the GPU's PCIe root (cross-socket DMA halves the
     # copy bandwidth and made the number swing run to run). Restored afterwards.
@@ -575,20 +666,33 @@ def _run_e2e(points, unit, args, device):
 
     main = torch.cuda.current_stream(device)
     streams = [torch.cuda.Stream(device=device) for _ in range(2)]
-    hx = [p.x.cpu().pin_memory() for p in points]
+    # host buffers: one pinned input / output per distinct shape (the host side has no L2 to defeat)
+    hx, hy = {}, {}
+    for p in points:
+        key = (p.kind, p.dims, p.K)
+        if p.kind == "single" and (p.dims, p.n_local) not in hx:
+            hx[(p.dims, p.n_local)] = p.x.cpu().pin_memory()
+        elif p.kind == "multi":
+            hx[key] = p.x.cpu().pin_memory()
+        hy[key] = torch.empty(tuple(p.y.shape), dtype=torch.float32, pin_memory=True)
     hf = [p.f.cpu().pin_memory() for p in points]
-    hy = [torch.empty(tuple(p.y.shape), dtype=torch.float32, pin_memory=True) for p in points]
     steps = max(1, min(args.steps, args.e2e_steps))
 
     def one():
         for s in streams:
             s.wait_stream(main)
+        c = 0
         for i, p in enumerate(points):
-            s = streams[i % 2]
+            key = (p.kind, p.dims, p.K)
             if p.kind == "single":
-                pkg.conv2d_single_host(hx[i], hf[i], device=device, stream=s, out_host=hy[i])
+                xin, yout = hx[(p.dims, p.n_local)], hy[key]
+                for j in range(p.n_local):
+                    pkg.conv2d_single_host(xin[j], hf[i], device=device, stream=streams[c % 2], out_host=yout[j])
+                    c += 1
             else:
-                pkg.conv2d_multi_host(hx[i], hf[i], device=device, stream=s, out_host=hy[i], impl=args.multi_impl)
+                pkg.conv2d_multi_host(hx[key], hf[i], device=device, stream=streams[c % 2], out_host=hy[key],
+                                      impl=args.multi_impl)
+                c += 1
         for s in streams:
             main.wait_stream(s)
 
@@ -602,13 +706,14 @@ def _run_e2e(points, unit, args, device):
     e1.record(main)
     torch.cuda.synchronize()
     ms = e0.elapsed_time(e1)
-    units = sum(p.out_px if unit == "Gpixel/s" else p.flops for p in points) * steps
-    h2d = sum(p.in_bytes() + p.filt_bytes() for p in points)
+    units = sum(p.local_units(unit) for p in points) * steps
+    h2d = sum(p.in_bytes() + p.filt_bytes() * (p.n_local if p.kind == "single" else 1) for p in points)
     d2h = sum(4 * p.y.numel() for p in points)
     return {"value": round(units / (ms * 1e-3) / 1e9, 3), "unit": unit, "h2d_bytes_per_step": h2d,
             "d2h_bytes_per_step": d2h, "steps": steps, "ms_per_step": round(ms / steps, 3),
-            "path": ("conv2d_single_host (C ABI, pinned host buffers, 2 streams)" if points[0].kind == "single"
-                     else f"conv2d_multi_host (impl={args.multi_impl}; pinned host buffers, 2 streams)")}
+            "path": ("conv2d_single_host (C ABI, pinned host buffers, one call per image, 2 streams)"
+                     if points[0].kind == "single" else
+                     f"conv2d_multi_host (impl={args.multi_impl}; pinned host buffers, 2 streams)")}
 
 
 def load_traffic(p):
@@ -677,11 +782,11 @@ def _calibrate(points, budget_s):
     return min(1.0, frac * budget_s / max(s, 1e-6)), u, s
 
 
-def cpu_baseline(workload, budget_s=10.0):
+def cpu_baseline(workload, budget_s=10.0, batch=None):
     _set_omp()
     import oracle
 
-    points, unit = workload_points(workload)
+    points, unit = workload_points(workload, batch)
     frac, _, _ = _calibrate(points, budget_s)
     u, s = _oracle_sample(points, frac)
     what = "output rows" if points[0].kind == "single" else "images"
@@ -698,7 +803,7 @@ def run_reference(args):
     _set_omp()
     import oracle
 
-    points, unit = workload_points(args.workload)
+    points, unit = workload_points(args.workload, args.batch)
     budget = max(0.5, args.ref_budget / max(1, args.steps + args.warmup))
     frac, _, _ = _calibrate(points, budget)
     for _ in range(args.warmup):
@@ -728,6 +833,20 @@ def run_reference(args):
     }), flush=True)
 
 
+def torchrun_cmd(argv, gpus, port):
+    """The command that re-launches this script with one process per GPU (the driver's own form)."""
+    return [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={gpus}",
+            "--master-addr", "127.0.0.1", f"--master-port={port}", os.path.abspath(__file__), *argv]
+
+
+def _free_port():
+    import socket
+
+    with socket.socket() as s:
+        s.bind(("127.0.0.1", 0))
+        return s.getsockname()[1]
+
+
 def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("--gpus", type=int, default=1)
@@ -735,7 +854,10 @@ def main():
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
     ap.add_argument("--workload", default="sweep", choices=sorted(WORKLOAD_DESC))
-    ap.add_argument("--e2e-steps", type=int, default=5)
+    ap.add_argument("--batch", type=int, default=None,
+                    help=f"images per single-channel point (sweep default {DEFAULT_SWEEP_BATCH}, config0 default 1); "
+                         "split across ranks")
+    ap.add_argument("--e2e-steps", type=int, default=3)
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--cpu-budget", type=float, default=10.0)
@@ -755,12 +877,23 @@ def main():
     args = ap.parse_args()
     if args.warmup < 3 and args.impl == "ours":
         args.warmup = 3  # contract: W >= 3
+    if args.batch is not None and args.batch < 1:
+        raise SystemExit("--batch must be >= 1")
     if args.workload in ("pad", "halo"):
         args.no_e2e = True  # the host-buffer entry (e2e) is the valid-mode one-segment call
     if args.impl == "reference":
         run_reference(args)
-    else:
-        run_ours(args)
+        return
+    if args.gpus > 1 and "WORLD_SIZE" not in os.environ:
+        # one process per GPU: re-launch under torchrun (the driver launches us that way itself)
+        import torch
+
+        have = torch.cuda.device_count()
+        if have < args.gpus:
+            raise SystemExit(f"bench.py: --gpus {args.gpus} needs {args.gpus} visible GPUs, found {have}")
+        cmd = torchrun_cmd(sys.argv[1:], args.gpus, _free_port())
+        os.execvp(cmd[0], cmd)
+    run_ours(args)
 
 
 if __name__ == "__main__":

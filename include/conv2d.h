@@ -81,6 +81,16 @@ int conv2d_multi(const float *in, int N, int C, int H, int W, const float *filt,
                  float *out, void *stream);
 
 /*
+ * A batch of N single-channel images filtered with one filter (image filtering of a batch; also the
+ * unit the multi-GPU bench shards across ranks): the same operation as N conv2d_single calls on
+ * in + n*H*W -> out + n*(H-K+1)*(W-K+1), n < N, in ONE launch (the warp tiles of all images form one
+ * wave, so small images fill the GPU). Same layouts, ownership, stream semantics, errors and bits as
+ * conv2d_single on each image (CONV2D_ESHAPE also for N < 1).
+ */
+int conv2d_single_batch(const float *in, int N, int H, int W, const float *filt, int K, float *out,
+                        void *stream);
+
+/*
  * Same as conv2d_single / conv2d_multi with an explicit output-row band height per warp
  * (band_h <= 0: the library's choice). For tuning sweeps and tests of the band / halo logic; the
  * result is bitwise identical for every band_h (each output's summation order does not depend on
@@ -182,7 +192,7 @@ int conv2d_release_scratch(void);
 /* Human-readable text for a return code (static storage, never NULL). */
 const char *conv2d_strerror(int code);
 
-/* ABI version (major*100 + minor). */
+/* ABI version (major*100 + minor): 102 = conv2d_single_batch. */
 int conv2d_version(void);
 
 #ifdef __cplusplus

@@ -9,9 +9,9 @@ The product is libconv2d.so (C ABI, include/conv2d.h). This package is its thin 
             memory or CUDA IPC mappings)
 """
 from . import _capi
-from .api import (conv2d_multi, conv2d_multi_host, conv2d_multi_tc, conv2d_single, conv2d_single_direct,
-                  conv2d_single_halo, conv2d_single_host, conv2d_single_pad)
+from .api import (conv2d_multi, conv2d_multi_host, conv2d_multi_tc, conv2d_single, conv2d_single_batch,
+                  conv2d_single_direct, conv2d_single_halo, conv2d_single_host, conv2d_single_pad)
 
 __all__ = ["_capi", "conv2d_multi", "conv2d_multi_host", "conv2d_multi_tc", "conv2d_single",
-           "conv2d_single_direct", "conv2d_single_halo", "conv2d_single_host",
+           "conv2d_single_batch", "conv2d_single_direct", "conv2d_single_halo", "conv2d_single_host",
            "conv2d_single_pad"]

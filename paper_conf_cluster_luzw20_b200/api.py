@@ -57,24 +57,62 @@ def _check_dev(t: torch.Tensor, name: str):
         raise ValueError(f"{name} must be contiguous")
 
 
+def _out_for(out, shape, like: torch.Tensor, name="out") -> torch.Tensor:
+    """The caller's `out` checked against the result shape (device, dtype, contiguity, same device as
+    the input) -- the C ABI cannot know the size of an output buffer -- or a new tensor."""
+    shape = tuple(int(v) for v in shape)
+    if out is None:
+        return torch.empty(shape, dtype=torch.float32, device=like.device)
+    _check_dev(out, name)
+    if out.device != like.device:
+        raise ValueError(f"{name} must be on {like.device}, got {out.device}")
+    if tuple(out.shape) != shape:
+        raise ValueError(f"{name} has shape {tuple(out.shape)}, expected {shape}")
+    return out
+
+
+def _check_same_device(*ts):
+    d = ts[0].device
+    for t in ts[1:]:
+        if t.device != d:
+            raise ValueError(f"all tensors must be on one device ({d} vs {t.device})")
+
+
 def conv2d_single(x: torch.Tensor, f: torch.Tensor, out: torch.Tensor | None = None, stream=None,
                   band_h: int = 0) -> torch.Tensor:
     _check_dev(x, "x")
     _check_dev(f, "f")
     if x.dim() != 2 or f.dim() != 2 or f.shape[0] != f.shape[1]:
         raise ValueError("x must be (H, W) and f (K, K)")
+    _check_same_device(x, f)
     H, W = x.shape
     K = f.shape[0]
-    if out is None:
-        out = torch.empty((max(H - K + 1, 0), max(W - K + 1, 0)), dtype=torch.float32, device=x.device)
-    else:
-        _check_dev(out, "out")
-        if tuple(out.shape) != (H - K + 1, W - K + 1):
-            raise ValueError("out has the wrong shape")
+    out = _out_for(out, (max(H - K + 1, 0), max(W - K + 1, 0)), x)
     dev = x.device.index
     with _on_device(dev):
         rc = _capi.lib().conv2d_single_ex(x.data_ptr(), H, W, f.data_ptr(), K, out.data_ptr(),
                                           _stream_handle(stream, dev), band_h)
+    if rc:
+        _capi.check(rc)
+    return out
+
+
+def conv2d_single_batch(x: torch.Tensor, f: torch.Tensor, out: torch.Tensor | None = None,
+                        stream=None) -> torch.Tensor:
+    """A batch of images (N, H, W) filtered with one filter f (K, K) in one launch -> (N, H-K+1, W-K+1);
+    bitwise equal to conv2d_single on every image. include/conv2d.h: conv2d_single_batch."""
+    _check_dev(x, "x")
+    _check_dev(f, "f")
+    if x.dim() != 3 or f.dim() != 2 or f.shape[0] != f.shape[1]:
+        raise ValueError("x must be (N, H, W) and f (K, K)")
+    _check_same_device(x, f)
+    N, H, W = x.shape
+    K = f.shape[0]
+    out = _out_for(out, (N, max(H - K + 1, 0), max(W - K + 1, 0)), x)
+    dev = x.device.index
+    with _on_device(dev):
+        rc = _capi.lib().conv2d_single_batch(x.data_ptr(), N, H, W, f.data_ptr(), K, out.data_ptr(),
+                                             _stream_handle(stream, dev))
     if rc:
         _capi.check(rc)
     return out
@@ -94,13 +132,8 @@ def conv2d_single_halo(x: torch.Tensor, halo: torch.Tensor, f: torch.Tensor, out
     H, W = x.shape
     Hh = halo.shape[0]
     K = f.shape[0]
-    shape = (max(H + Hh - K + 1, 0), max(W - K + 1, 0))
-    if out is None:
-        out = torch.empty(shape, dtype=torch.float32, device=x.device)
-    else:
-        _check_dev(out, "out")
-        if tuple(out.shape) != shape:
-            raise ValueError("out has the wrong shape")
+    _check_same_device(x, f)
+    out = _out_for(out, (max(H + Hh - K + 1, 0), max(W - K + 1, 0)), x)
     dev = x.device.index
     with _on_device(dev):
         _capi.check(_capi.conv2d_single_halo(x.data_ptr(), H, W, halo.data_ptr() if Hh else 0, Hh, f.data_ptr(), K,
@@ -123,15 +156,10 @@ def conv2d_single_pad(x: torch.Tensor, f: torch.Tensor, padding: str = "same", f
     if padding not in _PAD_MODES:
         raise ValueError(f"padding must be one of {sorted(_PAD_MODES)}")
     mode = _PAD_MODES[padding] | (_capi.CONV2D_FLIP if flip else 0)
+    _check_same_device(x, f)
     H, W = x.shape
     K = f.shape[0]
-    shape = (H, W) if mode & 3 else (max(H - K + 1, 0), max(W - K + 1, 0))
-    if out is None:
-        out = torch.empty(shape, dtype=torch.float32, device=x.device)
-    else:
-        _check_dev(out, "out")
-        if tuple(out.shape) != shape:
-            raise ValueError("out has the wrong shape")
+    out = _out_for(out, (H, W) if mode & 3 else (max(H - K + 1, 0), max(W - K + 1, 0)), x)
     dev = x.device.index
     with _on_device(dev):
         _capi.check(_capi.conv2d_single_pad(x.data_ptr(), H, W, f.data_ptr(), K, mode, out.data_ptr(),
@@ -144,10 +172,12 @@ def conv2d_single_direct(x: torch.Tensor, f: torch.Tensor, out: torch.Tensor | N
     """PAPER.md Fig. 1a baseline kernel (no column/row reuse); evidence control only."""
     _check_dev(x, "x")
     _check_dev(f, "f")
+    if x.dim() != 2 or f.dim() != 2 or f.shape[0] != f.shape[1]:
+        raise ValueError("x must be (H, W) and f (K, K)")
+    _check_same_device(x, f)
     H, W = x.shape
     K = f.shape[0]
-    if out is None:
-        out = torch.empty((H - K + 1, W - K + 1), dtype=torch.float32, device=x.device)
+    out = _out_for(out, (max(H - K + 1, 0), max(W - K + 1, 0)), x)
     dev = x.device.index
     with _on_device(dev):
         _capi.check(_capi.conv2d_single_direct(x.data_ptr(), H, W, f.data_ptr(), K, out.data_ptr(),
@@ -161,14 +191,10 @@ def conv2d_multi(x: torch.Tensor, w: torch.Tensor, out: torch.Tensor | None = No
     _check_dev(w, "w")
     if x.dim() != 4 or w.dim() != 4 or w.shape[1] != x.shape[1] or w.shape[2] != w.shape[3]:
         raise ValueError("x must be (N, C, H, W) and w (F, C, K, K)")
+    _check_same_device(x, w)
     N, C, H, W = x.shape
     F, _, K, _ = w.shape
-    if out is None:
-        out = torch.empty((N, F, max(H - K + 1, 0), max(W - K + 1, 0)), dtype=torch.float32, device=x.device)
-    else:
-        _check_dev(out, "out")
-        if tuple(out.shape) != (N, F, H - K + 1, W - K + 1):
-            raise ValueError("out has the wrong shape")
+    out = _out_for(out, (N, F, max(H - K + 1, 0), max(W - K + 1, 0)), x)
     dev = x.device.index
     with _on_device(dev):
         rc = _capi.lib().conv2d_multi_ex(x.data_ptr(), N, C, H, W, w.data_ptr(), F, K, out.data_ptr(),
@@ -184,10 +210,10 @@ def conv2d_multi_tc(x: torch.Tensor, w: torch.Tensor, out: torch.Tensor | None =
     _check_dev(w, "w")
     if x.dim() != 4 or w.dim() != 4 or w.shape[1] != x.shape[1] or w.shape[2] != w.shape[3]:
         raise ValueError("x must be (N, C, H, W) and w (F, C, K, K)")
+    _check_same_device(x, w)
     N, C, H, W = x.shape
     F, _, K, _ = w.shape
-    if out is None:
-        out = torch.empty((N, F, max(H - K + 1, 0), max(W - K + 1, 0)), dtype=torch.float32, device=x.device)
+    out = _out_for(out, (N, F, max(H - K + 1, 0), max(W - K + 1, 0)), x)
     dev = x.device.index
     with _on_device(dev):
         _capi.check(_capi.conv2d_multi_tc(x.data_ptr(), N, C, H, W, w.data_ptr(), F, K, out.data_ptr(),
@@ -204,12 +230,20 @@ def conv2d_single_host(x_host: torch.Tensor, f_host: torch.Tensor, device="cuda"
         raise TypeError("conv2d_single_host takes host tensors")
     if x_host.dtype != torch.float32 or f_host.dtype != torch.float32:
         raise TypeError("float32 tensors required")
+    if x_host.dim() != 2 or f_host.dim() != 2 or f_host.shape[0] != f_host.shape[1]:
+        raise ValueError("x_host must be (H, W) and f_host (K, K)")
     x_host = x_host.contiguous()
     f_host = f_host.contiguous()
     H, W = x_host.shape
     K = f_host.shape[0]
+    shape = (max(H - K + 1, 0), max(W - K + 1, 0))
     if out_host is None:
-        out_host = torch.empty((max(H - K + 1, 0), max(W - K + 1, 0)), dtype=torch.float32, pin_memory=True)
+        out_host = torch.empty(shape, dtype=torch.float32, pin_memory=True)
+    else:
+        if out_host.is_cuda or out_host.dtype != torch.float32 or not out_host.is_contiguous():
+            raise TypeError("out_host must be a contiguous float32 host tensor")
+        if tuple(out_host.shape) != shape:
+            raise ValueError(f"out_host has shape {tuple(out_host.shape)}, expected {shape}")
     dev = torch.device(device)
     s = stream if stream is not None else torch.cuda.current_stream(dev)
     with torch.cuda.device(dev):

@@ -11,9 +11,11 @@
 
 namespace c2d {
 
+#ifdef C2D_TUNING
 std::atomic<int> g_variant{0};
 std::atomic<int> g_min_band{0};
 std::atomic<int> g_mvariant{0};
+#endif
 
 // ------------------------------------------------------------------------------------------------
 // Baseline: PAPER.md Fig. 1a direct convolution, one thread per output, K*K loads per thread
@@ -78,8 +80,6 @@ namespace {
 
 using namespace c2d;
 
-constexpr int kMaxDevices = 64;
-
 DevInfo g_dev[kMaxDevices];
 std::once_flag g_dev_once[kMaxDevices];
 
@@ -87,6 +87,7 @@ int current_device_info(DevInfo *out) {
   int dev = 0;
   if (cudaGetDevice(&dev) != cudaSuccess || dev < 0 || dev >= kMaxDevices) return CONV2D_ECUDA;
   std::call_once(g_dev_once[dev], [dev] {
+    g_dev[dev].id = dev;
     cudaDeviceGetAttribute(&g_dev[dev].num_sms, cudaDevAttrMultiProcessorCount, dev);
     cudaDeviceGetAttribute(&g_dev[dev].smem_optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev);
   });
@@ -127,26 +128,38 @@ int check_k(int K) {
   return CONV2D_OK;
 }
 
+// Validation shared by the one-image and the batched call (N images of H x W, dense, back to back).
+int single_batch_impl(const float *in, int N, int H, int W, const float *filt, int K, float *out, void *stream,
+                      int band_h) {
+  if (!in || !filt || !out) return CONV2D_ENULL;
+  if (int e = check_k(K)) return e;
+  if (N < 1 || H < K || W < K) return CONV2D_ESHAPE;
+  if (!aligned4(in) || !aligned4(filt) || !aligned4(out)) return CONV2D_EALIGN;
+  const double in_n = static_cast<double>(N) * H * W;
+  if (in_n > 4.0e18 || static_cast<double>(N) * (H - K + 1) * (W - K + 1) * 1.0 > 4.0e18) return CONV2D_ESHAPE;
+  const size_t in_b = static_cast<size_t>(N) * H * W * sizeof(float);
+  const size_t out_b = static_cast<size_t>(N) * (H - K + 1) * (W - K + 1) * sizeof(float);
+  const size_t f_b = static_cast<size_t>(K) * K * sizeof(float);
+  if (overlap(in, in_b, out, out_b) || overlap(filt, f_b, out, out_b)) return CONV2D_EOVERLAP;
+  DevInfo dev;
+  if (current_device_info(&dev)) return CONV2D_ECUDA;
+  cudaStream_t s = static_cast<cudaStream_t>(stream);
+#define C2D_CALL_SINGLE(KK) single_entry<KK>(in, N, H, W, filt, out, s, band_h, dev, in, H, W, W - KK + 1)
+  C2D_K_SWITCH(K, C2D_CALL_SINGLE)
+#undef C2D_CALL_SINGLE
+}
+
 }  // namespace
 
 extern "C" {
 
 int conv2d_single_ex(const float *in, int H, int W, const float *filt, int K, float *out, void *stream,
                      int band_h) {
-  if (!in || !filt || !out) return CONV2D_ENULL;
-  if (int e = check_k(K)) return e;
-  if (H < K || W < K) return CONV2D_ESHAPE;
-  if (!aligned4(in) || !aligned4(filt) || !aligned4(out)) return CONV2D_EALIGN;
-  const size_t in_b = static_cast<size_t>(H) * W * sizeof(float);
-  const size_t out_b = static_cast<size_t>(H - K + 1) * (W - K + 1) * sizeof(float);
-  const size_t f_b = static_cast<size_t>(K) * K * sizeof(float);
-  if (overlap(in, in_b, out, out_b) || overlap(filt, f_b, out, out_b)) return CONV2D_EOVERLAP;
-  DevInfo dev;
-  if (current_device_info(&dev)) return CONV2D_ECUDA;
-  cudaStream_t s = static_cast<cudaStream_t>(stream);
-#define C2D_CALL_SINGLE(KK) single_entry<KK>(in, H, W, filt, out, s, band_h, dev, in, H, W, W - KK + 1)
-  C2D_K_SWITCH(K, C2D_CALL_SINGLE)
-#undef C2D_CALL_SINGLE
+  return single_batch_impl(in, 1, H, W, filt, K, out, stream, band_h);
+}
+
+int conv2d_single_batch(const float *in, int N, int H, int W, const float *filt, int K, float *out, void *stream) {
+  return single_batch_impl(in, N, H, W, filt, K, out, stream, 0);
 }
 
 int conv2d_single_halo(const float *in, int H, int W, const float *halo, int halo_rows, const float *filt, int K,
@@ -169,7 +182,7 @@ int conv2d_single_halo(const float *in, int H, int W, const float *halo, int hal
   if (current_device_info(&dev)) return CONV2D_ECUDA;
   cudaStream_t s = static_cast<cudaStream_t>(stream);
   const int Hi = static_cast<int>(Ht);
-#define C2D_CALL_HALO(KK) single_entry<KK>(in, Hi, W, filt, out, s, 0, dev, halo, H, W, W - KK + 1)
+#define C2D_CALL_HALO(KK) single_entry<KK>(in, 1, Hi, W, filt, out, s, 0, dev, halo, H, W, W - KK + 1)
   C2D_K_SWITCH(K, C2D_CALL_HALO)
 #undef C2D_CALL_HALO
 }
@@ -237,27 +250,21 @@ const char *conv2d_strerror(int code) {
   }
 }
 
-int conv2d_version(void) { return 101; }
+int conv2d_version(void) { return 102; }
 
 int conv2d_release_scratch(void) { return scratch_trim() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA; }
 
-// Not part of include/conv2d.h: selects a kernel variant for tuning tools (0 = default).
-int c2d_debug_set_variant(int v) {
-  const int old = g_variant.exchange(v);
-  return old;
-}
+#ifdef C2D_TUNING
+// Tuning build only (libconv2d_tune.so; not part of include/conv2d.h): force a kernel variant for
+// tuning tools and the variant tests (0 = default).
+int c2d_debug_set_variant(int v) { return g_variant.exchange(v); }
 
-// Not part of include/conv2d.h: multi-channel variant for tuning tools (0 = default; 1/2 constant
-// filters wide/narrow segments; 3/4 shared-memory filters wide/narrow; 9 = round-1 kernel).
-int c2d_debug_set_multi_variant(int v) {
-  const int old = g_mvariant.exchange(v);
-  return old;
-}
+// multi-channel variant (0 = default; 1/2 FB wide/narrow segments, 3/4 half FB, 5/6 two column chunks,
+// 7 8-lane segments, 9 = round-1 kernel)
+int c2d_debug_set_multi_variant(int v) { return g_mvariant.exchange(v); }
 
-// Not part of include/conv2d.h: minimum band height override for tuning tools (0 = default).
-int c2d_debug_set_min_band(int v) {
-  const int old = g_min_band.exchange(v);
-  return old;
-}
+// minimum band height override (0 = default)
+int c2d_debug_set_min_band(int v) { return g_min_band.exchange(v); }
+#endif
 
 }  // extern "C"

@@ -13,7 +13,7 @@
 
 namespace {
 
-constexpr int kMaxDevices = 64;
+using c2d::kMaxDevices;
 constexpr int kEvents = 64;  // event ring (per device)
 
 struct HostPipe {
@@ -40,14 +40,26 @@ extern "C" int conv2d_single_host(const float *in, int H, int W, const float *fi
   int dev = 0;
   if (cudaGetDevice(&dev) != cudaSuccess || dev < 0 || dev >= kMaxDevices) return CONV2D_ECUDA;
   HostPipe &p = g_pipe[dev];
-  std::lock_guard<std::mutex> lk(p.mu);
-  if (!p.init) {
-    if (cudaStreamCreateWithFlags(&p.s_in, cudaStreamNonBlocking) != cudaSuccess) return CONV2D_ECUDA;
-    if (cudaStreamCreateWithFlags(&p.s_out, cudaStreamNonBlocking) != cudaSuccess) return CONV2D_ECUDA;
-    for (int i = 0; i < kEvents; ++i)
-      if (cudaEventCreateWithFlags(&p.ev[i], cudaEventDisableTiming) != cudaSuccess) return CONV2D_ECUDA;
-    p.init = true;
+  {  // lazy init only; the copies and kernels below run without the lock (pageable copies block)
+    std::lock_guard<std::mutex> lk(p.mu);
+    if (!p.init) {
+      if (cudaStreamCreateWithFlags(&p.s_in, cudaStreamNonBlocking) != cudaSuccess) return CONV2D_ECUDA;
+      if (cudaStreamCreateWithFlags(&p.s_out, cudaStreamNonBlocking) != cudaSuccess) return CONV2D_ECUDA;
+      for (int i = 0; i < kEvents; ++i)
+        if (cudaEventCreateWithFlags(&p.ev[i], cudaEventDisableTiming) != cudaSuccess) return CONV2D_ECUDA;
+      p.init = true;
+    }
   }
+  // an event of the ring (a stream wait captures the event's state when it is enqueued, so an event
+  // re-recorded later by another call does not disturb an earlier wait)
+  auto next_event = [&p]() {
+    std::lock_guard<std::mutex> lk(p.mu);
+    return p.get();
+  };
+  auto link = [&](cudaStream_t from, cudaStream_t to) {  // `to` waits for the work enqueued on `from`
+    cudaEvent_t e = next_event();
+    return cudaEventRecord(e, from) == cudaSuccess && cudaStreamWaitEvent(to, e, 0) == cudaSuccess;
+  };
   cudaStream_t s = static_cast<cudaStream_t>(stream);
   const int Ho = H - K + 1, Wo = W - K + 1;
   if (chunk_rows <= 0) chunk_rows = std::max(1, static_cast<int>((8ll << 20) / (4ll * W)));
@@ -57,10 +69,7 @@ extern "C" int conv2d_single_host(const float *in, int H, int W, const float *fi
   const size_t f_b = static_cast<size_t>(K) * K * sizeof(float);
 
   // everything starts after the work already on `stream`
-  cudaEvent_t e0 = p.get();
-  if (cudaEventRecord(e0, s) != cudaSuccess) return CONV2D_ECUDA;
-  if (cudaStreamWaitEvent(p.s_in, e0, 0) != cudaSuccess) return CONV2D_ECUDA;
-  if (cudaStreamWaitEvent(p.s_out, e0, 0) != cudaSuccess) return CONV2D_ECUDA;
+  if (!link(s, p.s_in) || !link(s, p.s_out)) return CONV2D_ECUDA;
 
   void *d_buf = nullptr;
   const size_t in_pad = (in_b + 255) / 256 * 256, out_pad = (out_b + 255) / 256 * 256;
@@ -68,39 +77,42 @@ extern "C" int conv2d_single_host(const float *in, int H, int W, const float *fi
   float *d_in = static_cast<float *>(d_buf);
   float *d_out = reinterpret_cast<float *>(static_cast<char *>(d_buf) + in_pad);
   float *d_f = reinterpret_cast<float *>(static_cast<char *>(d_buf) + in_pad + out_pad);
-  if (cudaMemcpyAsync(d_f, filt, f_b, cudaMemcpyHostToDevice, p.s_in) != cudaSuccess) return CONV2D_ECUDA;
 
   int rc = CONV2D_OK;
+  if (cudaMemcpyAsync(d_f, filt, f_b, cudaMemcpyHostToDevice, p.s_in) != cudaSuccess) rc = CONV2D_ECUDA;
   int copied = 0;  // input rows already on the device
-  cudaEvent_t e_last_out = nullptr;
   for (int o0 = 0; o0 < Ho && rc == CONV2D_OK; o0 += chunk_rows) {
     const int rows = std::min(chunk_rows, Ho - o0);
     const int need = o0 + rows + K - 1;  // input rows [0, need) required for this chunk
     if (need > copied) {
       if (cudaMemcpyAsync(d_in + static_cast<size_t>(copied) * W, in + static_cast<size_t>(copied) * W,
                           static_cast<size_t>(need - copied) * W * sizeof(float), cudaMemcpyHostToDevice,
-                          p.s_in) != cudaSuccess)
-        return CONV2D_ECUDA;
+                          p.s_in) != cudaSuccess) {
+        rc = CONV2D_ECUDA;
+        break;
+      }
       copied = need;
     }
-    cudaEvent_t e_in = p.get();
-    if (cudaEventRecord(e_in, p.s_in) != cudaSuccess || cudaStreamWaitEvent(s, e_in, 0) != cudaSuccess)
-      return CONV2D_ECUDA;
+    if (!link(p.s_in, s)) {
+      rc = CONV2D_ECUDA;
+      break;
+    }
     rc = conv2d_single_ex(d_in + static_cast<size_t>(o0) * W, rows + K - 1, W, d_f, K,
                           d_out + static_cast<size_t>(o0) * Wo, s, 0);
     if (rc != CONV2D_OK) break;
-    cudaEvent_t e_k = p.get();
-    if (cudaEventRecord(e_k, s) != cudaSuccess || cudaStreamWaitEvent(p.s_out, e_k, 0) != cudaSuccess)
-      return CONV2D_ECUDA;
+    if (!link(s, p.s_out)) {
+      rc = CONV2D_ECUDA;
+      break;
+    }
     if (cudaMemcpyAsync(out + static_cast<size_t>(o0) * Wo, d_out + static_cast<size_t>(o0) * Wo,
                         static_cast<size_t>(rows) * Wo * sizeof(float), cudaMemcpyDeviceToHost,
                         p.s_out) != cudaSuccess)
-      return CONV2D_ECUDA;
+      rc = CONV2D_ECUDA;
   }
-  // release the buffer after the last D2H, and order `stream` after everything
-  e_last_out = p.get();
-  if (cudaEventRecord(e_last_out, p.s_out) != cudaSuccess) return CONV2D_ECUDA;
-  if (cudaStreamWaitEvent(s, e_last_out, 0) != cudaSuccess) return CONV2D_ECUDA;
-  if (cudaFreeAsync(d_buf, s) != cudaSuccess) return CONV2D_ECUDA;
+  // One exit path, also on errors: `stream` is ordered after everything enqueued on both copy
+  // streams (nothing keeps writing into the caller's buffers unordered), then the scratch buffer is
+  // released on `stream`.
+  const bool joined = link(p.s_in, s) && link(p.s_out, s);
+  if (cudaFreeAsync(d_buf, s) != cudaSuccess || !joined) return rc != CONV2D_OK ? rc : CONV2D_ECUDA;
   return rc;
 }

@@ -352,23 +352,29 @@ struct SingleArgs {
   const float *filt;
   float *out;
   int H, W, Ho, Wo;
-  int band_h;     // output rows per warp tile
-  int n_cb;       // column blocks of 128*U outputs
-  int n_tiles;    // n_cb * n_bands
-  int aligned;    // in is 16B aligned and W % 4 == 0
+  int n_img;          // images of a batch (conv2d_single_batch); image i at in + i*img_in, out + i*img_out
+  long long img_in;   // floats between consecutive input images (H * P)
+  long long img_out;  // floats between consecutive output images (Ho * Po)
+  int n_bands;        // output-row bands per image: band b = rows [b*Ho/n_bands, (b+1)*Ho/n_bands)
+  int n_cb;           // column blocks of 128*U outputs
+  int n_tiles;        // n_img * n_bands * n_cb
+  int aligned;        // in is 16B aligned and W % 4 == 0
 };
+
+// Output rows of band b of n (balanced: heights differ by at most one row, so a wave of n_bands
+// bands per column block is exactly n_bands tiles and no SM gets a short tile).
+__device__ __forceinline__ int band_start(int b, int n, int Ho) {
+  return static_cast<int>(static_cast<long long>(b) * Ho / n);
+}
 
 // HALO: rows >= H1 come from in2 (conv2d_single_halo); a separate instantiation, so the one-segment
 // kernels keep their row addressing (the per-row select measured -2% at K = 11..15).
 template <bool HALO>
-__device__ __forceinline__ const float *in_row(const SingleArgs &a, int r) {
+__device__ __forceinline__ const float *in_row(const SingleArgs &a, const float *__restrict__ inb, int r) {
   if constexpr (HALO)
-    return r < a.H1 ? a.in + static_cast<size_t>(r) * a.P : a.in2 + static_cast<size_t>(r - a.H1) * a.P;
+    return r < a.H1 ? inb + static_cast<size_t>(r) * a.P : a.in2 + static_cast<size_t>(r - a.H1) * a.P;
   else
-    return a.in + static_cast<size_t>(r) * a.P;
-}
-__device__ __forceinline__ float *out_row(const SingleArgs &a, int o) {
-  return a.out + static_cast<size_t>(o) * a.Po;
+    return inb + static_cast<size_t>(r) * a.P;
 }
 
 // One warp tile: 128*U columns x output rows [ob, oe). Input rows [ob, oe+K-1) stream through once,
@@ -388,7 +394,8 @@ __device__ __forceinline__ float *out_row(const SingleArgs &a, int o) {
 // PF 1/2: rows r+1 (r+2) in flight in registers; PF >= 3 (power of two, EDGE < 2): a PF-stage cp.async
 // ring in shared memory with PF-1 rows in flight (latency-bound short bands and HBM-bound small K).
 template <int K, int U, int FSRC, int PF, int GUARDS, int EDGE, bool HALO>
-__device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc<K, FSRC> &fs, int x0, int ob,
+__device__ __forceinline__ void single_tile(const SingleArgs &a, const float *__restrict__ inb,
+                                            float *__restrict__ outb, const FilterSrc<K, FSRC> &fs, int x0, int ob,
                                             int oe, int lane, unsigned ring_base) {
   constexpr bool SAFE = (EDGE != 0);
   constexpr int NST = (PF >= 3 && EDGE != 2) ? PF : 1;
@@ -411,10 +418,10 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc
   RowBuf<K, U> n1, n2;  // register path: rows r+1 (and r+2 when RPF == 2) in flight
   if constexpr (NST > 1) {
 #pragma unroll
-    for (int st = 0; st < NST - 1; ++st) ring.issue(st, in_row<HALO>(a, min(ob + st, rlast)), x0, a.Wc, clamp);
+    for (int st = 0; st < NST - 1; ++st) ring.issue(st, in_row<HALO>(a, inb, min(ob + st, rlast)), x0, a.Wc, clamp);
   } else {
-    load_row<K, U, SAFE>(n1, in_row<HALO>(a, ob), x0, a.Wc, lane, a.aligned);
-    if (RPF == 2) load_row<K, U, SAFE>(n2, in_row<HALO>(a, min(ob + 1, rlast)), x0, a.Wc, lane, a.aligned);
+    load_row<K, U, SAFE>(n1, in_row<HALO>(a, inb, ob), x0, a.Wc, lane, a.aligned);
+    if (RPF == 2) load_row<K, U, SAFE>(n2, in_row<HALO>(a, inb, min(ob + 1, rlast)), x0, a.Wc, lane, a.aligned);
   }
   // returns row r and issues the fetch of row r+depth (index clamped)
   auto next_row = [&](int r) {
@@ -423,14 +430,14 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc
       cp_async_wait<NST - 2>();
       const int k = r - ob;
       ring.read(k & (NST - 1), cur);
-      ring.issue((k + NST - 1) & (NST - 1), in_row<HALO>(a, min(r + NST - 1, rlast)), x0, a.Wc, clamp);
+      ring.issue((k + NST - 1) & (NST - 1), in_row<HALO>(a, inb, min(r + NST - 1, rlast)), x0, a.Wc, clamp);
     } else if constexpr (RPF == 2) {
       cur = n1;
       n1 = n2;
-      load_row<K, U, SAFE>(n2, in_row<HALO>(a, min(r + 2, rlast)), x0, a.Wc, lane, a.aligned);
+      load_row<K, U, SAFE>(n2, in_row<HALO>(a, inb, min(r + 2, rlast)), x0, a.Wc, lane, a.aligned);
     } else {
       cur = n1;
-      load_row<K, U, SAFE>(n1, in_row<HALO>(a, min(r + 1, rlast)), x0, a.Wc, lane, a.aligned);
+      load_row<K, U, SAFE>(n1, in_row<HALO>(a, inb, min(r + 1, rlast)), x0, a.Wc, lane, a.aligned);
     }
     return cur;
   };
@@ -441,7 +448,7 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc
       float w[U][KCfg<K>::WN];
       build_windows<K, U>(cur, w, lane);
       row_step1<K, U, FSRC, false>(acc, w, fs, 0, K);
-      if (r >= ob + K - 1) store_row<U, SAFE>(out_row(a, r - K + 1), x0, a.Wo, acc[0], lane);
+      if (r >= ob + K - 1) store_row<U, SAFE>(outb + static_cast<size_t>(r - K + 1) * a.Po, x0, a.Wo, acc[0], lane);
     }
     return;
   }
@@ -457,14 +464,14 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const FilterSrc
     float w[U][KCfg<K>::WN];
     build_windows<K, U>(cur, w, lane);
     row_step1<K, U, FSRC, false>(acc, w, fs, 0, K);
-    if (GUARDS == 2 || r >= ob + K - 1) store_row<U, SAFE>(out_row(a, r - K + 1), x0, a.Wo, acc[0], lane);
+    if (GUARDS == 2 || r >= ob + K - 1) store_row<U, SAFE>(outb + static_cast<size_t>(r - K + 1) * a.Po, x0, a.Wo, acc[0], lane);
   }
   for (; r < rend; ++r) {  // case 3 (GUARDS == 2): slots of outputs < oe only (>= ob for short bands)
     const RowBuf<K, U> cur = next_row(r);
     float w[U][KCfg<K>::WN];
     build_windows<K, U>(cur, w, lane);
     row_step1<K, U, FSRC, true>(acc, w, fs, max(0, K - 1 - (r - ob)), oe + K - 1 - r);
-    if (r >= ob + K - 1) store_row<U, SAFE>(out_row(a, r - K + 1), x0, a.Wo, acc[0], lane);
+    if (r >= ob + K - 1) store_row<U, SAFE>(outb + static_cast<size_t>(r - K + 1) * a.Po, x0, a.Wo, acc[0], lane);
   }
 }
 
@@ -494,18 +501,22 @@ __global__ void __launch_bounds__(CTAW *kWarp) k_conv2d_single(const SingleArgs 
   const unsigned ring_base = static_cast<unsigned>(__cvta_generic_to_shared(ring_smem)) +
                              warp * RowRing<K, U, kWarp, (PF >= 3 ? PF : 2)>::kBytes;
   const int cb = tile % a.n_cb;
-  const int band = tile / a.n_cb;
+  const int t2 = tile / a.n_cb;
+  const int band = t2 % a.n_bands;
+  const int img = t2 / a.n_bands;
+  const float *__restrict__ inb = a.in + img * a.img_in;
+  float *__restrict__ outb = a.out + img * a.img_out;
   const int x0 = cb * 128 * U;
-  const int ob = band * a.band_h;
-  const int oe = min(ob + a.band_h, a.Ho);
+  const int ob = band_start(band, a.n_bands, a.Ho);
+  const int oe = band_start(band + 1, a.n_bands, a.Ho);
   // fast tiles: 16B-aligned rows, every column of the tile and its extra halo quad in range
   const bool inside = x0 + 128 * U + 4 * KCfg<K>::NE <= a.W;  // warp-uniform
   if (a.aligned && inside)
-    single_tile<K, U, FSRC, PF, GUARDS, 0, HALO>(a, fs, x0, ob, oe, lane, ring_base);
+    single_tile<K, U, FSRC, PF, GUARDS, 0, HALO>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
   else if (a.aligned)
-    single_tile<K, U, FSRC, PF, GUARDS, 1, HALO>(a, fs, x0, ob, oe, lane, ring_base);
+    single_tile<K, U, FSRC, PF, GUARDS, 1, HALO>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
   else
-    single_tile<K, U, FSRC, PF, GUARDS, 2, HALO>(a, fs, x0, ob, oe, lane, ring_base);
+    single_tile<K, U, FSRC, PF, GUARDS, 2, HALO>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
 }
 
 // ------------------------------------------------------------------------------------------------

@@ -61,23 +61,39 @@ bool overlap(const void *a, size_t abytes, const void *b, size_t bbytes) {
   return a0 < b0 + bbytes && b0 < a0 + abytes;
 }
 
-// one non-blocking side stream per device for the border strips (created on first use, never freed)
-constexpr int kSideDevices = 64;
-std::mutex g_side_mu;
-cudaStream_t g_side[kSideDevices] = {};
+// Border-strip side stream and its fork / join events: one set per (host thread, device), created on
+// first use and kept, so concurrent callers on different threads never share a side stream.
+struct SideSet {
+  cudaStream_t stream = nullptr;
+  cudaEvent_t fork = nullptr, join = nullptr;
+  bool ok = false;
+};
+thread_local SideSet t_side[kMaxDevices];
 
-cudaStream_t side_stream() {
-  int dev = 0;
-  if (cudaGetDevice(&dev) != cudaSuccess || dev < 0 || dev >= kSideDevices) return nullptr;
-  std::lock_guard<std::mutex> lk(g_side_mu);
-  if (!g_side[dev] && cudaStreamCreateWithFlags(&g_side[dev], cudaStreamNonBlocking) != cudaSuccess)
-    g_side[dev] = nullptr;
-  return g_side[dev];
+SideSet *side_set(int dev) {
+  if (dev < 0 || dev >= kMaxDevices) return nullptr;
+  SideSet &ss = t_side[dev];
+  if (!ss.ok) {
+    if (cudaStreamCreateWithFlags(&ss.stream, cudaStreamNonBlocking) != cudaSuccess ||
+        cudaEventCreateWithFlags(&ss.fork, cudaEventDisableTiming) != cudaSuccess ||
+        cudaEventCreateWithFlags(&ss.join, cudaEventDisableTiming) != cudaSuccess) {
+      (void)cudaGetLastError();
+      return nullptr;
+    }
+    ss.ok = true;
+  }
+  return &ss;
+}
+
+bool capturing(cudaStream_t s) {
+  cudaStreamCaptureStatus st = cudaStreamCaptureStatusNone;
+  return cudaStreamIsCapturing(s, &st) == cudaSuccess && st != cudaStreamCaptureStatusNone;
 }
 
 int device_info(DevInfo *out) {
   int dev = 0;
   if (cudaGetDevice(&dev) != cudaSuccess) return CONV2D_ECUDA;
+  out->id = dev;
   if (cudaDeviceGetAttribute(&out->num_sms, cudaDevAttrMultiProcessorCount, dev) != cudaSuccess ||
       cudaDeviceGetAttribute(&out->smem_optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev) != cudaSuccess)
     return CONV2D_ECUDA;
@@ -129,7 +145,7 @@ extern "C" int conv2d_single_pad(const float *in, int H, int W, const float *fil
                      float *dst, int po) -> int {
     switch (K) {
 #define C2D_CALL_PAD(KK) \
-  case KK: return single_entry<KK>(src, rows, cols, f_use, dst, st, band_flag, dev, src, rows, pitch, po);
+  case KK: return single_entry<KK>(src, 1, rows, cols, f_use, dst, st, band_flag, dev, src, rows, pitch, po);
       C2D_CALL_PAD(1) C2D_CALL_PAD(2) C2D_CALL_PAD(3) C2D_CALL_PAD(4) C2D_CALL_PAD(5) C2D_CALL_PAD(6)
       C2D_CALL_PAD(7) C2D_CALL_PAD(8) C2D_CALL_PAD(9) C2D_CALL_PAD(10) C2D_CALL_PAD(11) C2D_CALL_PAD(12)
       C2D_CALL_PAD(13) C2D_CALL_PAD(14) C2D_CALL_PAD(15)
@@ -189,13 +205,13 @@ extern "C" int conv2d_single_pad(const float *in, int H, int W, const float *fil
   }
   int rc = CONV2D_OK;
   cudaStream_t ss = s;  // the strips' stream
-  cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
-  if (interior && ns > 0) {
-    cudaStream_t side = side_stream();
-    if (side && cudaEventCreateWithFlags(&ev_fork, cudaEventDisableTiming) == cudaSuccess &&
-        cudaEventCreateWithFlags(&ev_join, cudaEventDisableTiming) == cudaSuccess &&
-        cudaEventRecord(ev_fork, s) == cudaSuccess && cudaStreamWaitEvent(side, ev_fork, 0) == cudaSuccess)
-      ss = side;
+  SideSet *side = nullptr;
+  // Fork the strips onto this thread's side stream -- but not while `s` is being captured into a
+  // graph: a side stream forked from a capturing stream joins that capture, so the strips stay on `s`.
+  if (interior && ns > 0 && !capturing(s)) {
+    side = side_set(dev.id);
+    if (side && cudaEventRecord(side->fork, s) == cudaSuccess && cudaStreamWaitEvent(side->stream, side->fork, 0) == cudaSuccess)
+      ss = side->stream;
   }
   for (int t = 0; t < ns && rc == CONV2D_OK; ++t) {
     const Strip &st = strips[t];
@@ -213,11 +229,9 @@ extern "C" int conv2d_single_pad(const float *in, int H, int W, const float *fil
   }
   if (rc == CONV2D_OK && interior) rc = conv(in, H, W, W, out + static_cast<long long>(pt) * W + pl, W);
   if (ss != s) {  // join the strips back into the caller's stream (also on an error: nothing may dangle)
-    if (cudaEventRecord(ev_join, ss) != cudaSuccess || cudaStreamWaitEvent(s, ev_join, 0) != cudaSuccess)
+    if (cudaEventRecord(side->join, ss) != cudaSuccess || cudaStreamWaitEvent(s, side->join, 0) != cudaSuccess)
       rc = CONV2D_ECUDA;
   }
-  if (ev_fork) cudaEventDestroy(ev_fork);
-  if (ev_join) cudaEventDestroy(ev_join);
   if (scratch) cudaFreeAsync(scratch, s);
   if (f_rot) cudaFreeAsync(f_rot, s);
   return rc;

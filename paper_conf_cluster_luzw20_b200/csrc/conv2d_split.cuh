@@ -39,9 +39,12 @@ struct SplitArgs {
   int Po;       // output row pitch, as SingleArgs
   float *out;
   int H, W, Ho, Wo;
-  int band_h;   // output rows per cluster tile
+  int n_img;          // images of a batch, as SingleArgs
+  long long img_in;   // floats between consecutive input images
+  long long img_out;  // floats between consecutive output images
+  int n_bands;  // balanced output-row bands per image (band_start)
   int n_cb;     // column blocks of 128*U outputs
-  int n_tiles;  // n_cb * n_bands (clusters)
+  int n_tiles;  // n_img * n_bands * n_cb (clusters)
   int aligned;  // in is 16B aligned and W % 4 == 0
 };
 
@@ -123,8 +126,9 @@ struct SplitBuf {
 // named barrier). smem0: this CTA's dynamic shared memory; each part owns PW bytes of it (CL = 0: at
 // RANK * PW) holding its 3 chunk buffers and its row ring.
 template <int K, int G, int RANK, int U, int PF, int R, int GUARDS, int EDGE, int CL>
-__device__ __forceinline__ void split_tile(const SplitArgs &a, const FilterSrc<K, FSRC_CONST> &fs, int x0, int ob,
-                                           int oe, int lane, unsigned smem0, unsigned PW) {
+__device__ __forceinline__ void split_tile(const SplitArgs &a, const float *__restrict__ inb,
+                                           float *__restrict__ outb, const FilterSrc<K, FSRC_CONST> &fs, int x0,
+                                           int ob, int oe, int lane, unsigned smem0, unsigned PW) {
   constexpr int I0 = SplitRows<K, G, RANK>::I0;
   constexpr int KG = SplitRows<K, G, RANK>::KG;
   constexpr bool SAFE = (EDGE != 0);
@@ -171,7 +175,7 @@ __device__ __forceinline__ void split_tile(const SplitArgs &a, const FilterSrc<K
   constexpr bool clamp = (EDGE == 1);
   RowBuf<K, U> n1;
   auto in_row_p = [&](int r) {
-    return r < a.H1 ? a.in + static_cast<size_t>(r) * a.P : a.in2 + static_cast<size_t>(r - a.H1) * a.P;
+    return r < a.H1 ? inb + static_cast<size_t>(r) * a.P : a.in2 + static_cast<size_t>(r - a.H1) * a.P;
   };
   if constexpr (NST > 1) {
 #pragma unroll
@@ -221,7 +225,7 @@ __device__ __forceinline__ void split_tile(const SplitArgs &a, const FilterSrc<K
           }
         }
       }
-      float *orow = a.out + static_cast<size_t>(ob + c * R + k) * a.Po;
+      float *orow = outb + static_cast<size_t>(ob + c * R + k) * a.Po;
       store_row<U, SAFE>(orow, x0, a.Wo, o, lane);
     }
   };
@@ -256,13 +260,14 @@ __device__ __forceinline__ void split_tile(const SplitArgs &a, const FilterSrc<K
 }
 
 template <int K, int G, int U, int PF, int R, int GUARDS, int EDGE, int CL, int RK = 0>
-__device__ __forceinline__ void split_dispatch(unsigned rank, const SplitArgs &a, const FilterSrc<K, FSRC_CONST> &fs,
+__device__ __forceinline__ void split_dispatch(unsigned rank, const SplitArgs &a, const float *__restrict__ inb,
+                                               float *__restrict__ outb, const FilterSrc<K, FSRC_CONST> &fs,
                                                int x0, int ob, int oe, int lane, unsigned smem0, unsigned PW) {
   if constexpr (RK < G) {
     if (rank == RK)
-      split_tile<K, G, RK, U, PF, R, GUARDS, EDGE, CL>(a, fs, x0, ob, oe, lane, smem0, PW);
+      split_tile<K, G, RK, U, PF, R, GUARDS, EDGE, CL>(a, inb, outb, fs, x0, ob, oe, lane, smem0, PW);
     else
-      split_dispatch<K, G, U, PF, R, GUARDS, EDGE, CL, RK + 1>(rank, a, fs, x0, ob, oe, lane, smem0, PW);
+      split_dispatch<K, G, U, PF, R, GUARDS, EDGE, CL, RK + 1>(rank, a, inb, outb, fs, x0, ob, oe, lane, smem0, PW);
   }
 }
 
@@ -284,17 +289,21 @@ __global__ void __launch_bounds__(CL ? kWarp : G * kWarp) k_conv2d_split(const S
   const unsigned smem0 = static_cast<unsigned>(__cvta_generic_to_shared(split_smem));
   constexpr unsigned PW = SplitSmem<K, U, PF, R>::kPart;
   const int cb = tile % a.n_cb;
-  const int band = tile / a.n_cb;
+  const int t2 = tile / a.n_cb;
+  const int band = t2 % a.n_bands;
+  const int img = t2 / a.n_bands;
+  const float *__restrict__ inb = a.in + img * a.img_in;
+  float *__restrict__ outb = a.out + img * a.img_out;
   const int x0 = cb * 128 * U;
-  const int ob = band * a.band_h;
-  const int oe = min(ob + a.band_h, a.Ho);
+  const int ob = band_start(band, a.n_bands, a.Ho);
+  const int oe = band_start(band + 1, a.n_bands, a.Ho);
   const bool inside = x0 + 128 * U + 4 * KCfg<K>::NE <= a.W;  // uniform over the cluster
   if (a.aligned && inside)
-    split_dispatch<K, G, U, PF, R, GUARDS, 0, CL>(rank, a, fs, x0, ob, oe, lane, smem0, PW);
+    split_dispatch<K, G, U, PF, R, GUARDS, 0, CL>(rank, a, inb, outb, fs, x0, ob, oe, lane, smem0, PW);
   else if (a.aligned)
-    split_dispatch<K, G, U, PF, R, GUARDS, 1, CL>(rank, a, fs, x0, ob, oe, lane, smem0, PW);
+    split_dispatch<K, G, U, PF, R, GUARDS, 1, CL>(rank, a, inb, outb, fs, x0, ob, oe, lane, smem0, PW);
   else
-    split_dispatch<K, G, U, PF, R, GUARDS, 2, CL>(rank, a, fs, x0, ob, oe, lane, smem0, PW);
+    split_dispatch<K, G, U, PF, R, GUARDS, 2, CL>(rank, a, inb, outb, fs, x0, ob, oe, lane, smem0, PW);
 }
 
 }  // namespace c2d

@@ -27,6 +27,7 @@
 //     "empty" barriers, warp 9 lane 0 produces B. Global loads of K blocks kb+1 and kb+2 are in
 //     flight in registers while block kb is split and stored.
 //   * Epilogue: tcgen05.ld (each warp its 32 TMEM lanes) -> NFHoWo stores, coalesced along pixels.
+#include <atomic>
 #include <cstdint>
 
 #include <cuda_runtime.h>
@@ -677,14 +678,23 @@ __global__ void __launch_bounds__(TcPWarps<GW>::kThreads, 1) k_conv2d_multi_tc5(
   }
 }
 
-// Enable the dynamic shared memory a kernel instantiation may use (once per instantiation).
+// Enable the dynamic shared memory a kernel instantiation may use, once per instantiation and DEVICE
+// (cudaFuncSetAttribute acts on the current device only; a process may drive several GPUs).
+struct MaxDyn {
+  std::atomic<int> v[c2d::kMaxDevices] = {};
+};
 template <typename KernelT>
-int enable_smem(KernelT kernel, int &max_dyn) {
-  if (max_dyn > 0) return CONV2D_OK;
-  int dev = 0, optin = 0;
+int enable_smem(KernelT kernel, MaxDyn &cache, int *max_dyn) {
+  int dev = 0;
+  if (cudaGetDevice(&dev) != cudaSuccess || dev < 0 || dev >= c2d::kMaxDevices) return CONV2D_ECUDA;
+  const int known = cache.v[dev].load(std::memory_order_acquire);
+  if (known > 0) {
+    *max_dyn = known;
+    return CONV2D_OK;
+  }
+  int optin = 0;
   cudaFuncAttributes fa;
-  if (cudaGetDevice(&dev) != cudaSuccess ||
-      cudaDeviceGetAttribute(&optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev) != cudaSuccess ||
+  if (cudaDeviceGetAttribute(&optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev) != cudaSuccess ||
       cudaFuncGetAttributes(&fa, kernel) != cudaSuccess) {
     (void)cudaGetLastError();
     return CONV2D_ECUDA;
@@ -694,7 +704,8 @@ int enable_smem(KernelT kernel, int &max_dyn) {
     (void)cudaGetLastError();
     return CONV2D_ECUDA;
   }
-  max_dyn = avail;
+  cache.v[dev].store(avail, std::memory_order_release);
+  *max_dyn = avail;
   return CONV2D_OK;
 }
 
@@ -725,8 +736,9 @@ int launch_tc_d(TcArgs a, const float *filt, cudaStream_t stream) {
   using Cfg = TcCfg<FN, NBS, NACC>;
   auto kernel = k_conv2d_multi_tc4<FN, D, NBS, NACC>;
   const size_t smem = static_cast<size_t>(Cfg::NSB) * Cfg::kBStage + static_cast<size_t>(a.n_kb) * kKB * sizeof(int);
-  static int max_dyn = 0;
-  if (enable_smem(kernel, max_dyn) != CONV2D_OK) return CONV2D_ECUDA;
+  static MaxDyn smem_cache;
+  int max_dyn = 0;
+  if (enable_smem(kernel, smem_cache, &max_dyn) != CONV2D_OK) return CONV2D_ECUDA;
   if (smem > static_cast<size_t>(max_dyn)) return CONV2D_ESHAPE;
   return with_split_filters<FN>(a, filt, stream, [&](const float *bs, int n_fb) {
     a.bs = bs;
@@ -742,8 +754,9 @@ int launch_tc_p(TcArgs a, const float *filt, cudaStream_t stream) {
   using Cfg = TcPCfg<FN>;
   auto kernel = k_conv2d_multi_tc5<FN, D, GW>;
   const size_t smem = static_cast<size_t>(Cfg::NSB) * Cfg::kBStage + static_cast<size_t>(a.n_kb) * kKB * sizeof(int);
-  static int max_dyn = 0;
-  if (enable_smem(kernel, max_dyn) != CONV2D_OK) return CONV2D_ECUDA;
+  static MaxDyn smem_cache;
+  int max_dyn = 0;
+  if (enable_smem(kernel, smem_cache, &max_dyn) != CONV2D_OK) return CONV2D_ECUDA;
   if (smem > static_cast<size_t>(max_dyn)) return CONV2D_ESHAPE;
   int dev = 0, n_sm = 0;
   if (cudaGetDevice(&dev) != cudaSuccess || cudaDeviceGetAttribute(&n_sm, cudaDevAttrMultiProcessorCount, dev) != cudaSuccess)
@@ -758,18 +771,17 @@ int launch_tc_p(TcArgs a, const float *filt, cudaStream_t stream) {
   });
 }
 
-// Default: the persistent kernel. Tuning overrides (c2d_debug_set_multi_variant): 40 = one CTA per
-// tile (k_conv2d_multi_tc4, register ring depth 2), 23 / 24 = that with depth 3 / 4, 32-34 = with a
-// B ring of 2-4 stages.
+// Default: one CTA per (pixel tile, filter block), register ring depth 2, B ring of 2 stages. Tuning
+// build only (c2d_debug_set_multi_variant): 41 / 42 = two accumulators (B ring 2 / 3), 23 / 24 = ring
+// depth 3 / 4, 33 / 34 = a B ring of 3 / 4 stages, 50-55 = the persistent kernel (k_conv2d_multi_tc5).
 template <int FN>
 int launch_tc(const TcArgs &a, const float *filt, cudaStream_t stream) {
-  const int mv = c2d::g_mvariant.load(std::memory_order_relaxed);
-  if (mv == 40) return launch_tc_d<FN, 2, 2>(a, filt, stream);
+#ifdef C2D_TUNING
+  const int mv = c2d::tuning_mvariant();
   if (mv == 41) return launch_tc_d<FN, 2, 2, 2>(a, filt, stream);
   if (mv == 42) return launch_tc_d<FN, 2, 3, 2>(a, filt, stream);
   if (mv == 23) return launch_tc_d<FN, 3>(a, filt, stream);
   if (mv == 24) return launch_tc_d<FN, 4>(a, filt, stream);
-  if (mv == 32) return launch_tc_d<FN, 2, 2>(a, filt, stream);
   if (mv == 33) return launch_tc_d<FN, 2, 3>(a, filt, stream);
   if (mv == 34) return launch_tc_d<FN, 2, 4>(a, filt, stream);
   if (mv == 50) return launch_tc_p<FN, 2, 8>(a, filt, stream);
@@ -778,6 +790,7 @@ int launch_tc(const TcArgs &a, const float *filt, cudaStream_t stream) {
   if (mv == 53) return launch_tc_p<FN, 2, 16>(a, filt, stream);
   if (mv == 54) return launch_tc_p<FN, 3, 16>(a, filt, stream);
   if (mv == 55) return launch_tc_p<FN, 4, 16>(a, filt, stream);
+#endif
   return launch_tc_d<FN, 2, 2>(a, filt, stream);
 }
 
@@ -795,6 +808,13 @@ extern "C" int conv2d_multi_tc(const float *in, int N, int C, int H, int W, cons
   // 32-bit in-image offsets (one image's C planes) and a bounded im2col offset table
   if (static_cast<long long>(C) * H * W >= (1LL << 31) || static_cast<long long>(C) * K * K > (1 << 14))
     return CONV2D_ESHAPE;
+  {  // the output may overlap neither the input nor the filters (as conv2d_multi)
+    const uintptr_t o0 = reinterpret_cast<uintptr_t>(out);
+    const uintptr_t o1 = o0 + static_cast<size_t>(N) * F * (H - K + 1) * (W - K + 1) * sizeof(float);
+    const uintptr_t i0 = reinterpret_cast<uintptr_t>(in), i1 = i0 + static_cast<size_t>(N) * C * H * W * sizeof(float);
+    const uintptr_t f0 = reinterpret_cast<uintptr_t>(filt), f1 = f0 + static_cast<size_t>(F) * C * K * K * sizeof(float);
+    if ((o0 < i1 && i0 < o1) || (o0 < f1 && f0 < o1)) return CONV2D_EOVERLAP;
+  }
   TcArgs a;
   a.in = in;
   a.bs = nullptr;

@@ -2,8 +2,8 @@
 #include "launch.cuh"
 
 namespace c2d {
-template int single_entry<11>(const float *, int, int, const float *, float *, cudaStream_t, int, const DevInfo &,
-                                   const float *, int, long long, int);
+template int single_entry<11>(const float *, int, int, int, const float *, float *, cudaStream_t, int,
+                              const DevInfo &, const float *, int, long long, int);
 template int multi_entry<11>(const float *, int, int, int, int, const float *, int, float *, cudaStream_t, int,
                              const DevInfo &);
 }  // namespace c2d

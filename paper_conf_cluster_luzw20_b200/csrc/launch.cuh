@@ -19,33 +19,77 @@ namespace {
 
 using namespace c2d;
 
-constexpr int kMaxDevices = 64;
-
 bool aligned16(const void *p) { return (reinterpret_cast<uintptr_t>(p) & 15u) == 0; }
 
 int ceil_div(long long a, long long b) { return static_cast<int>((a + b - 1) / b); }
 
-// Occupancy (CTAs per SM) of a kernel instantiation, cached per instantiation (devices of one box
-// are identical B200s).
+// Occupancy (CTAs per SM) of one kernel instantiation, cached per dynamic shared-memory size (the
+// devices of one box are identical B200s; the smem size depends on call arguments such as C). A few
+// lock-free entries (smem << 16 | value); a miss past the last entry just recomputes.
+struct OccCache {
+  std::atomic<long long> e[8] = {};
+};
 template <typename KernelT>
-int cta_occupancy(KernelT kernel, size_t dyn_smem, std::atomic<int> &cache, int cta_warps = kCtaWarps) {
-  int v = cache.load(std::memory_order_relaxed);
-  if (v > 0) return v;
+int cta_occupancy(KernelT kernel, size_t dyn_smem, OccCache &cache, int cta_threads) {
+  const long long key = static_cast<long long>(dyn_smem) << 16;
+  for (auto &slot : cache.e) {
+    const long long v = slot.load(std::memory_order_relaxed);
+    if (v == 0) break;
+    if ((v & ~0xffffLL) == key) return static_cast<int>(v & 0xffff);
+  }
   int blocks = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, kernel, cta_warps * kWarp, dyn_smem) != cudaSuccess ||
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, kernel, cta_threads, dyn_smem) != cudaSuccess ||
       blocks < 1)
     blocks = 1;
-  cache.store(blocks, std::memory_order_relaxed);
+  for (auto &slot : cache.e) {
+    long long expect = 0;
+    if (slot.compare_exchange_strong(expect, key | blocks, std::memory_order_relaxed)) break;
+    if ((expect & ~0xffffLL) == key) break;
+  }
   return blocks;
+}
+
+// Opt a kernel instantiation into more than 48 KiB of dynamic shared memory, once per DEVICE (the
+// attribute is per device; a process may drive several GPUs).
+struct SmemOptIn {
+  std::atomic<int> done[kMaxDevices] = {};
+};
+template <typename KernelT>
+int ensure_smem(KernelT kernel, size_t smem, const DevInfo &dev, SmemOptIn &flag) {
+  if (smem <= 48 * 1024) return CONV2D_OK;
+  if (smem > static_cast<size_t>(dev.smem_optin)) return CONV2D_ESHAPE;
+  if (dev.id < 0 || dev.id >= kMaxDevices) return CONV2D_ECUDA;
+  if (flag.done[dev.id].load(std::memory_order_acquire)) return CONV2D_OK;
+  if (cudaFuncSetAttribute(kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, dev.smem_optin) != cudaSuccess)
+    return CONV2D_ECUDA;
+  flag.done[dev.id].store(1, std::memory_order_release);
+  return CONV2D_OK;
+}
+
+// Band count per image: one full wave of `resident` warp tiles over n_img images x n_cb column blocks,
+// bands at least min_band rows tall; band_h > 0 (explicit): ceil(Ho / band_h) bands. Bands are
+// balanced (band_start), so the wave is exactly filled.
+int band_count(int Ho, int n_cb, int n_img, long long resident, int band_h, int min_band) {
+  long long bands;
+  if (band_h > 0) {
+    bands = (Ho + static_cast<long long>(band_h) - 1) / band_h;
+  } else {
+    bands = resident / (static_cast<long long>(n_cb) * n_img);
+    const long long max_bands = min_band > 1 ? Ho / min_band : Ho;
+    if (bands > max_bands) bands = max_bands;
+  }
+  if (bands < 1) bands = 1;
+  if (bands > Ho) bands = Ho;
+  return static_cast<int>(bands);
 }
 
 // ------------------------------------------------------------------------------------------------
 // single channel
 // ------------------------------------------------------------------------------------------------
-// Variant override for tuning tools (c2d_debug_set_variant; 0 = the tuned default):
+// Tuning build only (c2d_debug_set_variant; 0 = the tuned default):
 //   1: filter in shared memory, U=1 (4 warps/CTA)     2: shared memory, U=2
 //   3: filter in a __constant__ slot, U=1 (1 warp/CTA) 4: __constant__ slot, U=2
-//   5-9, 13: guard / prefetch variants of the constant-slot kernel (see launch_single)
+//   5-9, 13, 15: guard / prefetch variants of the constant-slot kernel (see launch_single)
 //   10-12: filter-row split over G parts (conv2d_split.cuh)
 
 // Constant-bank filter slot of this unit (this K), per device: it holds the filter of the last call
@@ -62,10 +106,9 @@ struct ConstRing {
 ConstRing g_cring[kMaxDevices];
 
 template <typename LaunchFn>
-int with_const_filter(const float *filt, int K, int KP, cudaStream_t stream, LaunchFn launch) {
-  int dev = 0;
-  if (cudaGetDevice(&dev) != cudaSuccess || dev < 0 || dev >= kMaxDevices) return CONV2D_ECUDA;
-  ConstRing &ring = g_cring[dev];
+int with_const_filter(const float *filt, int K, int KP, cudaStream_t stream, const DevInfo &dev, LaunchFn launch) {
+  if (dev.id < 0 || dev.id >= kMaxDevices) return CONV2D_ECUDA;
+  ConstRing &ring = g_cring[dev.id];
   std::lock_guard<std::mutex> lk(ring.mu);
   if (!ring.init) {
     void *p = nullptr;
@@ -90,46 +133,56 @@ bool stream_capturing(cudaStream_t s) {
   return cudaStreamIsCapturing(s, &st) == cudaSuccess && st != cudaStreamCaptureStatusNone;
 }
 
+// Geometry shared by the one-warp-tile and the split launches.
+struct SingleGeom {
+  const float *in, *in2;
+  int N, H, W, H1;
+  long long P;
+  int Po;
+};
+
+template <typename ArgsT>
+void fill_args(ArgsT &a, const SingleGeom &g, int K, int U, float *out) {
+  a.in = g.in;
+  a.in2 = g.in2;
+  a.H1 = g.H1;
+  a.P = static_cast<int>(g.P);
+  a.Wc = static_cast<int>(g.P);
+  a.Po = g.Po;
+  a.out = out;
+  a.H = g.H;
+  a.W = g.W;
+  a.Ho = g.H - K + 1;
+  a.Wo = g.W - K + 1;
+  a.n_img = g.N;
+  a.img_in = static_cast<long long>(g.H) * g.P;
+  a.img_out = static_cast<long long>(a.Ho) * g.Po;
+  a.n_cb = ceil_div(a.Wo, 128 * U);
+  a.aligned = (aligned16(g.in) && aligned16(g.in2) && (g.P % 4 == 0)) ? 1 : 0;
+}
+
 template <int K, int U, int FSRC, int PF = 1, int GUARDS = 0, bool HALO = false>
-int launch_single_v(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                    const DevInfo &dev, int min_band, const float *in2, int H1, long long P, int Po) {
+int launch_single_v(const SingleGeom &g, const float *filt, float *out, cudaStream_t stream, int band_h,
+                    const DevInfo &dev, int min_band) {
   constexpr int CTAW = (FSRC == FSRC_CONST) ? 1 : kCtaWarps;
   auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS, HALO>;
-  static std::atomic<int> occ_cache{0};
+  static OccCache occ_cache;
   const size_t ring = (PF >= 3) ? CTAW * RowRing<K, U, kWarp, (PF >= 3 ? PF : 2)>::kBytes : 0;
   SingleArgs a;
-  a.in = in;
-  a.in2 = in2;
-  a.H1 = H1;
-  a.P = static_cast<int>(P);
-  a.Wc = static_cast<int>(P);
-  a.Po = Po;
+  fill_args(a, g, K, U, out);
   a.filt = filt;
-  a.out = out;
-  a.H = H;
-  a.W = W;
-  a.Ho = H - K + 1;
-  a.Wo = W - K + 1;
-  a.n_cb = ceil_div(a.Wo, 128 * U);
-  a.aligned = (aligned16(in) && aligned16(in2) && (P % 4 == 0)) ? 1 : 0;
-  if (band_h <= 0) {
-    // one full wave of warp tiles: bands = resident warps / column blocks
-    const long long resident_warps =
-        static_cast<long long>(cta_occupancy(kernel, ring, occ_cache, CTAW)) * CTAW * dev.num_sms;
-    const long long bands = resident_warps / a.n_cb > 0 ? resident_warps / a.n_cb : 1;
-    band_h = ceil_div(a.Ho, bands);
-    if (band_h < min_band) band_h = min_band;
-  }
-  if (band_h > a.Ho) band_h = a.Ho;
-  a.band_h = band_h;
-  const int n_bands = ceil_div(a.Ho, band_h);
-  a.n_tiles = a.n_cb * n_bands;
+  const long long resident = static_cast<long long>(cta_occupancy(kernel, ring, occ_cache, CTAW * kWarp)) * CTAW *
+                             dev.num_sms;
+  a.n_bands = band_count(a.Ho, a.n_cb, a.n_img, resident, band_h, min_band);
+  const long long tiles = static_cast<long long>(a.n_cb) * a.n_bands * a.n_img;
+  if (tiles > 0x7fffffffLL - CTAW) return CONV2D_ESHAPE;
+  a.n_tiles = static_cast<int>(tiles);
   const int blocks = ceil_div(a.n_tiles, CTAW);
   auto go = [&]() {
     kernel<<<blocks, CTAW * kWarp, ring, stream>>>(a);
     return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
   };
-  if constexpr (FSRC == FSRC_CONST) return with_const_filter(filt, K, KCfg<K>::KP, stream, go);
+  if constexpr (FSRC == FSRC_CONST) return with_const_filter(filt, K, KCfg<K>::KP, stream, dev, go);
   return go();
 }
 
@@ -137,34 +190,17 @@ int launch_single_v(const float *in, int H, int W, const float *filt, float *out
 // warps -- a cluster of G one-warp CTAs (CL = 1) or one CTA of G warps (CL = 0) -- so a full wave has
 // G times fewer, taller bands.
 template <int K, int G, int U, int PF, int R, int GUARDS, int CL>
-int launch_split_v(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                   const DevInfo &dev, int min_band, const float *in2, int H1, long long P, int Po) {
+int launch_split_v(const SingleGeom &g, const float *filt, float *out, cudaStream_t stream, int band_h,
+                   const DevInfo &dev, int min_band) {
   static_assert(G >= 1 && G <= 8 && G <= K, "portable cluster of at most K CTAs");
   auto kernel = k_conv2d_split<K, G, U, PF, R, GUARDS, CL>;
-  static std::atomic<int> occ_cache{0};
+  static OccCache occ_cache;  // CL = 1: resident clusters per GPU; CL = 0: CTAs per SM
+  static SmemOptIn smem_flag;
   const size_t smem = static_cast<size_t>(SplitSmem<K, U, PF, R>::kPart) * (CL ? 1 : G);
   const int threads = CL ? kWarp : G * kWarp;
   SplitArgs a;
-  a.in = in;
-  a.in2 = in2;
-  a.H1 = H1;
-  a.P = static_cast<int>(P);
-  a.Wc = static_cast<int>(P);
-  a.Po = Po;
-  a.out = out;
-  a.H = H;
-  a.W = W;
-  a.Ho = H - K + 1;
-  a.Wo = W - K + 1;
-  a.n_cb = ceil_div(a.Wo, 128 * U);
-  a.aligned = (aligned16(in) && aligned16(in2) && (P % 4 == 0)) ? 1 : 0;
-  static std::atomic<int> smem_set{0};
-  if (smem > 48 * 1024 && smem_set.load() == 0) {
-    if (smem > static_cast<size_t>(dev.smem_optin)) return CONV2D_ESHAPE;
-    if (cudaFuncSetAttribute(kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, dev.smem_optin) != cudaSuccess)
-      return CONV2D_ECUDA;
-    smem_set.store(1);
-  }
+  fill_args(a, g, K, U, out);
+  if (int e = ensure_smem(kernel, smem, dev, smem_flag)) return e;
   cudaLaunchConfig_t cfg = {};
   cfg.blockDim = dim3(threads, 1, 1);
   cfg.dynamicSmemBytes = smem;
@@ -176,10 +212,15 @@ int launch_split_v(const float *in, int H, int W, const float *filt, float *out,
   attr[0].val.clusterDim.z = 1;
   cfg.attrs = attr;
   cfg.numAttrs = CL ? 1 : 0;
+  long long resident = 1;
   if (band_h <= 0) {
     // resident tiles of one full wave (clusters: as the cluster scheduler places them)
-    int v = occ_cache.load(std::memory_order_relaxed);
-    if (v <= 0) {
+    int v = 0;
+    const long long key = static_cast<long long>(smem) << 16;
+    const long long cached = occ_cache.e[0].load(std::memory_order_relaxed);
+    if (cached != 0 && (cached & ~0xffffLL) == key) {
+      v = static_cast<int>(cached & 0xffff);
+    } else {
       if constexpr (CL) {
         cfg.gridDim = dim3(G * dev.num_sms, 1, 1);
         int clusters = 0;
@@ -192,16 +233,12 @@ int launch_split_v(const float *in, int H, int W, const float *filt, float *out,
           blocks = 1;
         v = blocks * dev.num_sms;
       }
-      occ_cache.store(v, std::memory_order_relaxed);
+      occ_cache.e[0].store(key | v, std::memory_order_relaxed);
     }
-    const long long bands = v / a.n_cb > 0 ? v / a.n_cb : 1;
-    band_h = ceil_div(a.Ho, bands);
-    if (band_h < min_band) band_h = min_band;
+    resident = v;
   }
-  if (band_h > a.Ho) band_h = a.Ho;
-  a.band_h = band_h;
-  const int n_bands = ceil_div(a.Ho, band_h);
-  const long long tiles = static_cast<long long>(a.n_cb) * n_bands;
+  a.n_bands = band_count(a.Ho, a.n_cb, a.n_img, resident, band_h, min_band);
+  const long long tiles = static_cast<long long>(a.n_cb) * a.n_bands * a.n_img;
   if (tiles * G > 0x7fffffffLL) return CONV2D_ESHAPE;
   a.n_tiles = static_cast<int>(tiles);
   cfg.gridDim = dim3(static_cast<unsigned>(CL ? tiles * G : tiles), 1, 1);
@@ -212,19 +249,17 @@ int launch_split_v(const float *in, int H, int W, const float *filt, float *out,
     }
     return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
   };
-  return with_const_filter(filt, K, KCfg<K>::KP, stream, go);
+  return with_const_filter(filt, K, KCfg<K>::KP, stream, dev, go);
 }
 
 // The tuned default kernel choice (HALO: conv2d_single_halo's two-segment row addressing, same choice
 // and so the same bits as the one-segment call on the concatenated rows).
 template <int K, bool HALO>
-int launch_single_default(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream,
-                          int band_h, const DevInfo &dev, const float *in2, int H1, long long P, int Po,
-                          int min_band, bool constant_ok) {
-#define C2D_LS(UU, FS, PFF, G) \
-  launch_single_v<K, UU, FS, PFF, G, HALO>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1, P, Po)
-#define C2D_SP(GG, UU, PFF, RR, CLL) \
-  launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(in, H, W, filt, out, stream, band_h, dev, 1, in2, H1, P, Po)
+int launch_single_default(const SingleGeom &g, const float *filt, float *out, cudaStream_t stream, int band_h,
+                          const DevInfo &dev, int min_band, bool constant_ok) {
+#define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G, HALO>(g, filt, out, stream, band_h, dev, min_band)
+#define C2D_SP(GG, UU, PFF, RR, CLL) launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(g, filt, out, stream, band_h, dev, 1)
+  const int W = g.W;
   const bool force_smem = band_h == kBandSmemFilter;
   const bool no_split = band_h == kBandNoSplit || force_smem;  // internal callers: the one-tile kernel's bits
   if (no_split) band_h = 0;
@@ -248,10 +283,12 @@ int launch_single_default(const float *in, int H, int W, const float *filt, floa
   // skips the constant-slot staging (a stream-ordered copy plus two event operations, ~3 us of host
   // and device time per call, tools/host_overhead.py). Same summation order, same bits.
   // (tools/small_sizes2.py, back-to-back calls: 1024^2 K=3 12.1 -> 8.0 us, K=5 12.0 -> 10.3 us)
-  const long long px = static_cast<long long>(H) * W;
+  const long long px = static_cast<long long>(g.H) * W * g.N;
   const bool small = px <= 512LL * 512 || (K <= 5 && px <= 1024LL * 1024);
-  if (!constant_ok || force_smem || (K < 11 && small))
-    return (K <= 7) ? C2D_LS(2, FSRC_SMEM, 1, 0) : C2D_LS(1, FSRC_SMEM, 1, 0);
+  if (!constant_ok || force_smem || (K < 11 && small)) {
+    if constexpr (K <= 7) return C2D_LS(2, FSRC_SMEM, 1, 0);
+    else return C2D_LS(1, FSRC_SMEM, 1, 0);
+  }
   if constexpr (K <= 5) {
     if (K <= 3 && W > 1024) return C2D_LS(2, FSRC_CONST, 1, 0);
     return C2D_LS(2, FSRC_CONST, 4, 0);
@@ -276,22 +313,21 @@ int launch_single_default(const float *in, int H, int W, const float *filt, floa
 }
 
 template <int K>
-int launch_single(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                  const DevInfo &dev, const float *in2, int H1, long long P, int Po) {
-  const int mb = g_min_band.load(std::memory_order_relaxed);
+int launch_single(const SingleGeom &g, const float *filt, float *out, cudaStream_t stream, int band_h,
+                  const DevInfo &dev) {
+  const int mb = tuning_min_band();
   // Minimum band height K-1 (>= 4) bounds the Alg. 2 case-1 overhead once a wave is full; images up
   // to 512^2 cannot fill a wave even with one-row bands, and there the latency of a band's row chain
   // dominates: no minimum (tools/latency.py, one 256^2 call: K=3 10.3 -> 8.9 us, K=9 20.7 -> 14.2 us,
   // K=15 smem path 42 -> 28.6 us). Band height never changes the bits.
-  const bool tiny = static_cast<long long>(H) * W <= 512LL * 512;
+  const bool tiny = static_cast<long long>(g.H) * g.W * g.N <= 512LL * 512;
   const int min_band = mb > 0 ? mb : (tiny ? 1 : (K - 1 > 4 ? K - 1 : 4));
-  const int v = g_variant.load(std::memory_order_relaxed);
   // CUDA-graph capture cannot use the event-guarded constant slots: shared-memory filter there
   const bool constant_ok = !stream_capturing(stream);
-  if (H1 < H) return launch_single_default<K, true>(in, H, W, filt, out, stream, band_h, dev, in2, H1, P, Po, min_band,
-                                                    constant_ok);
-#define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G>(in, H, W, filt, out, stream, band_h, dev, min_band, in2, H1, P, Po)
-  switch (v) {
+  if (g.H1 < g.H) return launch_single_default<K, true>(g, filt, out, stream, band_h, dev, min_band, constant_ok);
+#ifdef C2D_TUNING
+#define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G>(g, filt, out, stream, band_h, dev, min_band)
+  switch (tuning_variant()) {
     case 1: return C2D_LS(1, FSRC_SMEM, 1, 0);
     case 2: return C2D_LS(2, FSRC_SMEM, 1, 0);
     case 3: if (constant_ok) return C2D_LS(1, FSRC_CONST, 1, 0); break;
@@ -305,9 +341,10 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
     case 15: if constexpr (K >= 10) { if (constant_ok) return C2D_LS(1, FSRC_CONST, 4, 1); } break;
     default: break;
   }
+#undef C2D_LS
   // filter-row split (conv2d_split.cuh; variants 10-12)
-#define C2D_SP(GG, UU, PFF, RR, CLL) \
-  launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(in, H, W, filt, out, stream, band_h, dev, 1, in2, H1, P, Po)
+#define C2D_SP(GG, UU, PFF, RR, CLL) launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(g, filt, out, stream, band_h, dev, 1)
+  const int v = tuning_variant();
   if (constant_ok && v >= 10 && v <= 12) {
     if constexpr (K >= 3) {
       switch (v) {
@@ -318,9 +355,9 @@ int launch_single(const float *in, int H, int W, const float *filt, float *out, 
       }
     }
   }
-  return launch_single_default<K, false>(in, H, W, filt, out, stream, band_h, dev, in2, H1, P, Po, min_band,
-                                         constant_ok);
-#undef C2D_LS
+#undef C2D_SP
+#endif
+  return launch_single_default<K, false>(g, filt, out, stream, band_h, dev, min_band, constant_ok);
 }
 
 // ------------------------------------------------------------------------------------------------
@@ -335,13 +372,9 @@ template <int K, int FB>
 int launch_multi_fb(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
                     cudaStream_t stream, int band_h, const DevInfo &dev, size_t smem) {
   auto kernel = k_conv2d_multi<K, FB>;
-  static std::atomic<int> occ_cache{0};
-  static std::atomic<int> smem_set{0};
-  if (smem > 48 * 1024 && smem_set.load() < static_cast<int>(smem)) {
-    if (cudaFuncSetAttribute(kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, dev.smem_optin) != cudaSuccess)
-      return CONV2D_ECUDA;
-    smem_set.store(dev.smem_optin);
-  }
+  static OccCache occ_cache;
+  static SmemOptIn smem_flag;
+  if (int e = ensure_smem(kernel, smem, dev, smem_flag)) return e;
   MultiArgs a;
   a.in = in;
   a.filt = filt;
@@ -357,10 +390,9 @@ int launch_multi_fb(const float *in, int N, int C, int H, int W, const float *fi
   a.n_fb = ceil_div(F, FB);
   a.aligned = (aligned16(in) && (W % 4 == 0)) ? 1 : 0;
   if (band_h <= 0) {
-    // occupancy of this instantiation with this smem size (the cache holds the value for the
-    // first smem size seen; good enough for choosing a band height)
+    // occupancy of this instantiation with this smem size
     const long long resident_warps =
-        static_cast<long long>(cta_occupancy(kernel, smem, occ_cache)) * kCtaWarps * dev.num_sms;
+        static_cast<long long>(cta_occupancy(kernel, smem, occ_cache, kCtaWarps * kWarp)) * kCtaWarps * dev.num_sms;
     const long long groups = static_cast<long long>(N) * a.n_fb * a.n_cb;
     long long bands = resident_warps / groups;
     if (bands < 1) bands = 1;
@@ -387,16 +419,11 @@ int launch_multi2_v(const float *in, int N, int C, int H, int W, const float *fi
   constexpr int KP = KCfg<K>::KP;
   constexpr int SEGS = kWarp / SEG;
   auto kernel = k_conv2d_multi2<K, FB, U, SEG, GUARDS, PF>;
-  static std::atomic<int> occ_cache{0};
-  static std::atomic<int> smem_set{0};
+  static OccCache occ_cache;
+  static SmemOptIn smem_flag;
   const size_t ring = (PF >= 3) ? kCtaWarps * RowRing<K, U, SEG, PF>::kBytes : 0;
   const size_t smem = static_cast<size_t>(C) * K * FB * KP * sizeof(float) + ring;
-  if (smem > static_cast<size_t>(dev.smem_optin)) return CONV2D_ESHAPE;
-  if (smem > 48 * 1024 && smem_set.load() == 0) {
-    if (cudaFuncSetAttribute(kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, dev.smem_optin) != cudaSuccess)
-      return CONV2D_ECUDA;
-    smem_set.store(1);
-  }
+  if (int e = ensure_smem(kernel, smem, dev, smem_flag)) return e;
   Multi2Args a;
   a.in = in;
   a.filt = filt;
@@ -416,7 +443,7 @@ int launch_multi2_v(const float *in, int N, int C, int H, int W, const float *fi
     // one full wave of resident warps (tools/multi_band_sweep.py: for K >= 5 the K-1 prologue rows
     // of extra bands cost more than the wave quantisation they remove -- Table I CONV3/CONV5, configs[3])
     const long long resident_warps =
-        static_cast<long long>(cta_occupancy(kernel, smem, occ_cache)) * kCtaWarps * dev.num_sms;
+        static_cast<long long>(cta_occupancy(kernel, smem, occ_cache, kCtaWarps * kWarp)) * kCtaWarps * dev.num_sms;
     const long long groups = static_cast<long long>(a.n_groups) * a.n_fb * a.n_cb;
     long long bands = resident_warps / groups;
     if (bands < 1) bands = 1;
@@ -427,7 +454,7 @@ int launch_multi2_v(const float *in, int N, int C, int H, int W, const float *fi
     // that minimises waves(b) * (ceil(Ho / b) + K - 1). (One band per tile whenever the (image,
     // F-block, column-block) groups alone exceed a wave left e.g. Table I CONV11 at 1.15 waves -- 2
     // waves, the second 15% full: 946 -> 570 us; CONV8/9 2x.)
-    const long long resident_ctas = static_cast<long long>(cta_occupancy(kernel, smem, occ_cache)) * dev.num_sms;
+    const long long resident_ctas = static_cast<long long>(cta_occupancy(kernel, smem, occ_cache, kCtaWarps * kWarp)) * dev.num_sms;
     const long long groups = static_cast<long long>(a.n_groups) * a.n_fb;
     long long best_b = 1;
     double best = 1e300;
@@ -468,44 +495,49 @@ int launch_multi(const float *in, int N, int C, int H, int W, const float *filt,
   // FB filters per warp (K*FB*4 accumulators); FBH = half of it (more warps, smaller loop body)
   constexpr int FB = (K <= 3) ? 8 : (K <= 7 ? 4 : 2);
   constexpr int FBH = (FB > 1) ? FB / 2 : 1;
+  // the tuned default: FB = 8 filters per warp for K <= 3, half the register-limited FB above
+  constexpr int FBD = (K <= 3) ? FB : FBH;
   constexpr int GUARDS = (K <= 5) ? 2 : 0;
   constexpr int KP = KCfg<K>::KP;
   const int Wo = W - K + 1;
-  const int mv = g_mvariant.load(std::memory_order_relaxed);
+  const int mv = tuning_mvariant();
   int rc = CONV2D_ESHAPE;
+  // row prefetch: a 4-stage cp.async ring in shared memory for K >= 5; two entries in registers for
+  // K <= 3, where a (row, channel) entry carries few FMAs and the ring's per-entry cost dominates
+  constexpr int PF = (K <= 3) ? 2 : 4;
+#define C2D_LM(FBB, SEGG) \
+  launch_multi2_v<K, FBB, 1, SEGG, GUARDS, PF>(in, N, C, H, W, filt, F, out, stream, band_h, dev)
+#ifdef C2D_TUNING
+#define C2D_LM2(FBB, SEGG) \
+  launch_multi2_v<K, FBB, 2, SEGG, GUARDS, PF>(in, N, C, H, W, filt, F, out, stream, band_h, dev)
   if (mv == 9) {  // the round-1 kernel
     constexpr int LFB = MultiCfg<K>::FB;
     const size_t lsmem = static_cast<size_t>(C) * K * LFB * KP * sizeof(float);
     if (lsmem <= static_cast<size_t>(dev.smem_optin))
       return launch_multi_fb<K, LFB>(in, N, C, H, W, filt, F, out, stream, band_h, dev, lsmem);
   }
-  // row prefetch: a 4-stage cp.async ring in shared memory for K >= 5; two entries in registers for
-  // K <= 3, where a (row, channel) entry carries few FMAs and the ring's per-entry cost dominates
-  constexpr int PF = (K <= 3) ? 2 : 4;
-#define C2D_LM(FBB, SEGG) \
-  launch_multi2_v<K, FBB, 1, SEGG, GUARDS, PF>(in, N, C, H, W, filt, F, out, stream, band_h, dev)
-#define C2D_LM2(FBB, SEGG) \
-  launch_multi2_v<K, FBB, 2, SEGG, GUARDS, PF>(in, N, C, H, W, filt, F, out, stream, band_h, dev)
   constexpr int FBQ = (FBH > 1) ? FBH / 2 : 1;
   if (mv == 5) return C2D_LM2(FBH, 16);
   if (mv == 6) return C2D_LM2(FBQ, 16);
+  if (mv == 1) return C2D_LM(FB, 32);
+  if (mv == 2) return C2D_LM(FB, 16);
+  if (mv == 3) return C2D_LM(FBH, 32);
+  if (mv == 4) return C2D_LM(FBH, 16);
+  if (mv == 7) return (K > 3) ? C2D_LM(FBH, 8) : C2D_LM(FB, 8);
+#undef C2D_LM2
+#endif
   // Tuned on B200 (tools/multi_variants.py): 16-lane segments (two images per warp) unless they waste
   // clearly more lanes than whole-warp rows -- more column blocks take the vector fast path and the
-  // ragged edge is a smaller share; FB = 8 filters per warp for K <= 3, half the register-limited FB
-  // above (smaller loop body, more resident warps).
-  const bool seg16 = (mv == 2 || mv == 4) || (mv == 0 && N >= 2 && lane_use(Wo, 64) >= lane_use(Wo, 128) - 0.05);
+  // ragged edge is a smaller share.
+  const bool seg16 = mv == 0 && N >= 2 && lane_use(Wo, 64) >= lane_use(Wo, 128) - 0.05;
   // 8-lane segments (four images per warp, 32 columns each) for narrow layers: Table I's 8-26-column
   // outputs use 25-81% of the lanes instead of 12-41% (tools/multi_band_sweep.py)
-  const bool seg8 = mv == 7 || (mv == 0 && N >= 4 && Wo <= 32 && lane_use(Wo, 32) >= lane_use(Wo, 64) + 0.15);
-  const bool half = (mv == 3 || mv == 4) || (mv == 0 && K > 3);
+  const bool seg8 = mv == 0 && N >= 4 && Wo <= 32 && lane_use(Wo, 32) >= lane_use(Wo, 64) + 0.15;
   if (seg8)
-    rc = half ? C2D_LM(FBH, 8) : C2D_LM(FB, 8);
-  else if (half)
-    rc = seg16 ? C2D_LM(FBH, 16) : C2D_LM(FBH, 32);
+    rc = C2D_LM(FBD, 8);
   else
-    rc = seg16 ? C2D_LM(FB, 16) : C2D_LM(FB, 32);
+    rc = seg16 ? C2D_LM(FBD, 16) : C2D_LM(FBD, 32);
 #undef C2D_LM
-#undef C2D_LM2
   if (rc != CONV2D_ESHAPE) return rc;
   // F-block does not fit shared memory: round-1 kernel with one filter per warp
   const size_t smem1 = static_cast<size_t>(C) * K * KP * sizeof(float);
@@ -519,9 +551,10 @@ int launch_multi(const float *in, int N, int C, int H, int W, const float *filt,
 namespace c2d {
 
 template <int K>
-int single_entry(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream, int band_h,
-                 const DevInfo &dev, const float *in2, int H1, long long P, int Po) {
-  return launch_single<K>(in, H, W, filt, out, stream, band_h, dev, in2, H1, P, Po);
+int single_entry(const float *in, int N, int H, int W, const float *filt, float *out, cudaStream_t stream,
+                 int band_h, const DevInfo &dev, const float *in2, int H1, long long P, int Po) {
+  const SingleGeom g{in, in2, N, H, W, H1, P, Po};
+  return launch_single<K>(g, filt, out, stream, band_h, dev);
 }
 
 template <int K>

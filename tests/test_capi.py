@@ -117,3 +117,31 @@ def test_product_path_has_no_oracle_dependency():
                 src = open(os.path.join(dirpath, fn)).read()
                 assert "import oracle" not in src and "from oracle" not in src, fn
                 assert "liboracle" not in src and "conv2d_oracle" not in src, fn
+
+
+def test_batch_argument_errors_need_no_gpu(lib):
+    from paper_conf_cluster_luzw20_b200 import _capi as c
+
+    a, b, o = 0x10000, 0x20000000, 0x40000000  # fake, never dereferenced
+    assert c.conv2d_single_batch(None, 2, 8, 8, b, 3, o) == c.CONV2D_ENULL
+    assert c.conv2d_single_batch(a, 0, 8, 8, b, 3, o) == c.CONV2D_ESHAPE
+    assert c.conv2d_single_batch(a, 2, 8, 8, b, 16, o) == c.CONV2D_EK
+    assert c.conv2d_single_batch(a, 2, 2, 8, b, 3, o) == c.CONV2D_ESHAPE
+    # the second image's input (bytes 256..512) overlaps the output
+    assert c.conv2d_single_batch(a, 2, 8, 8, b, 3, a + 300) == c.CONV2D_EOVERLAP
+    assert c.conv2d_multi_tc(a, 2, 2, 8, 8, b, 1, 3, a + 100) == c.CONV2D_EOVERLAP
+
+
+def test_product_library_has_no_tuning_switches(lib):
+    """The shipped libconv2d.so exports exactly the header's C ABI (no process-global tuning
+    switches); the c2d_debug_set_* switches live in the separate tuning build libconv2d_tune.so."""
+    from paper_conf_cluster_luzw20_b200 import _capi
+
+    out = subprocess.run(["nm", "-D", "--defined-only", _capi.LIB_PATH], capture_output=True, text=True).stdout
+    exported = set(re.findall(r"\bT (\w+)$", out, flags=re.M))
+    c_linkage = {e for e in exported if not e.startswith("_Z")}  # C++ symbols are not the C ABI
+    assert c_linkage == set(_capi.EXPORTS), c_linkage ^ set(_capi.EXPORTS)
+    assert not any("debug" in e for e in exported)
+    out = subprocess.run(["nm", "-D", "--defined-only", _capi.TUNE_LIB_PATH], capture_output=True, text=True).stdout
+    for f in ("c2d_debug_set_variant", "c2d_debug_set_multi_variant", "c2d_debug_set_min_band"):
+        assert re.search(rf"\bT {f}$", out, flags=re.M), f

@@ -336,3 +336,26 @@ def test_halo_segment_bitwise(cuda_device, K):
                                     y.data_ptr()) == _capi.CONV2D_ESHAPE
     assert _capi.conv2d_single_halo(x.data_ptr(), 30, 64, halo.data_ptr(), K, _filt(K).data_ptr(), K,
                                     halo.data_ptr()) == _capi.CONV2D_EOVERLAP
+
+
+@pytest.mark.parametrize("K", [1, 3, 5, 7, 11, 15])
+def test_single_batch_equals_per_image(cuda_device, K):
+    """conv2d_single_batch (one launch over N images; the bench's sharding unit): bitwise equal to
+    conv2d_single on every image, every output against the oracle, for small images (one wave holds
+    all of them), narrow images with large K (filter-row split kernel), ragged and misaligned widths."""
+    for (N, H, W) in [(5, K + 40, 300), (3, K + 90, 1030), (9, K + 7, 129), (2, 2 * K + 200, 1024), (1, K + 5, 77)]:
+        x = dev_image((N, H, W), "img", seed=N * 100 + K)
+        f = _filt(K, "rand", seed=K)
+        y = pkg.conv2d_single_batch(x, f)
+        torch.cuda.synchronize()
+        for n in range(N):
+            assert torch.equal(y[n], pkg.conv2d_single(x[n], f)), (K, N, H, W, n)
+        xh, fh, yh = x.cpu().numpy(), f.cpu().numpy(), y.cpu().numpy()
+        for n in range(N):
+            check_full_single_host(xh[n], fh, yh[n])
+    xi = dev_image((4, K + 30, 260), "int", seed=K)
+    fi = _filt(K, "int", seed=K)
+    yi = pkg.conv2d_single_batch(xi, fi)
+    for n in range(4):
+        check_full_single(xi[n], fi, yi[n], exact=True)
+
