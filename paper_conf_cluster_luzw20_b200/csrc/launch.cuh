@@ -14,6 +14,7 @@
 #include "conv2d_kernels.cuh"
 #include "conv2d_multi.cuh"
 #include "conv2d_split.cuh"
+#include "conv2d_wide.cuh"
 
 namespace {
 
@@ -66,21 +67,35 @@ int ensure_smem(KernelT kernel, size_t smem, const DevInfo &dev, SmemOptIn &flag
   return CONV2D_OK;
 }
 
-// Band count per image: one full wave of `resident` warp tiles over n_img images x n_cb column blocks,
-// bands at least min_band rows tall; band_h > 0 (explicit): ceil(Ho / band_h) bands. Bands are
-// balanced (band_start), so the wave is exactly filled.
-int band_count(int Ho, int n_cb, int n_img, long long resident, int band_h, int min_band) {
-  long long bands;
+// Band count per image. band_h > 0 (explicit): ceil(Ho / band_h) bands. Automatic: a wave-quantisation
+// cost model over the n_img x n_cb x bands tiles with `resident` tiles per wave: a tile of h output
+// rows streams h + K - 1 input rows (Alg. 2 case 1 is K-1 rows of prologue), and the grid runs in
+// ceil(tiles / resident) waves, so pick the band count b minimising waves(b) * (ceil(Ho / b) + K - 1)
+// with bands at least min_band rows tall. (One image: one full wave of bands, the round-1 choice; a
+// batch of large images: several waves of taller bands instead of an under-filled single wave --
+// 8 x 8192^2 K=15: 4 bands per image filled 86% of one wave.) Bands are balanced (band_start).
+int band_count(int Ho, int K, int n_cb, int n_img, long long resident, int band_h, int min_band) {
   if (band_h > 0) {
-    bands = (Ho + static_cast<long long>(band_h) - 1) / band_h;
-  } else {
-    bands = resident / (static_cast<long long>(n_cb) * n_img);
-    const long long max_bands = min_band > 1 ? Ho / min_band : Ho;
-    if (bands > max_bands) bands = max_bands;
+    long long b = (Ho + static_cast<long long>(band_h) - 1) / band_h;
+    return static_cast<int>(b < 1 ? 1 : (b > Ho ? Ho : b));
   }
-  if (bands < 1) bands = 1;
-  if (bands > Ho) bands = Ho;
-  return static_cast<int>(bands);
+  const long long groups = static_cast<long long>(n_cb) * n_img;
+  long long bmax = min_band > 1 ? Ho / min_band : Ho;
+  if (bmax < 1) bmax = 1;
+  if (bmax > 8192) bmax = 8192;
+  if (resident < 1) resident = 1;
+  long long best_b = 1;
+  double best = 1e300;
+  for (long long b = 1; b <= bmax; ++b) {
+    const long long h = (Ho + b - 1) / b;
+    const long long waves = (groups * b + resident - 1) / resident;
+    const double cost = static_cast<double>(waves) * static_cast<double>(h + K - 1);
+    if (cost < best * (1.0 - 1e-9)) {  // ties: the fewest bands
+      best = cost;
+      best_b = b;
+    }
+  }
+  return static_cast<int>(best_b);
 }
 
 // ------------------------------------------------------------------------------------------------
@@ -173,13 +188,37 @@ int launch_single_v(const SingleGeom &g, const float *filt, float *out, cudaStre
   a.filt = filt;
   const long long resident = static_cast<long long>(cta_occupancy(kernel, ring, occ_cache, CTAW * kWarp)) * CTAW *
                              dev.num_sms;
-  a.n_bands = band_count(a.Ho, a.n_cb, a.n_img, resident, band_h, min_band);
+  a.n_bands = band_count(a.Ho, K, a.n_cb, a.n_img, resident, band_h, min_band);
   const long long tiles = static_cast<long long>(a.n_cb) * a.n_bands * a.n_img;
   if (tiles > 0x7fffffffLL - CTAW) return CONV2D_ESHAPE;
   a.n_tiles = static_cast<int>(tiles);
   const int blocks = ceil_div(a.n_tiles, CTAW);
   auto go = [&]() {
     kernel<<<blocks, CTAW * kWarp, ring, stream>>>(a);
+    return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
+  };
+  if constexpr (FSRC == FSRC_CONST) return with_const_filter(filt, K, KCfg<K>::KP, stream, dev, go);
+  return go();
+}
+
+// Wide-lane kernel (conv2d_wide.cuh): 8 contiguous columns per lane, 256-column warp tiles, one warp
+// per CTA.
+template <int K, int FSRC, int PF, int GUARDS, bool HALO = false>
+int launch_wide_v(const SingleGeom &g, const float *filt, float *out, cudaStream_t stream, int band_h,
+                  const DevInfo &dev, int min_band) {
+  auto kernel = k_conv2d_wide<K, FSRC, PF, GUARDS, HALO>;
+  static OccCache occ_cache;
+  const size_t ring = (PF >= 3) ? WideRing<K, (PF >= 3 ? PF : 2)>::kBytes : 0;
+  SingleArgs a;
+  fill_args(a, g, K, 2, out);  // n_cb in 256-column blocks (= two 128-column chunks)
+  a.filt = filt;
+  const long long resident = static_cast<long long>(cta_occupancy(kernel, ring, occ_cache, kWarp)) * dev.num_sms;
+  a.n_bands = band_count(a.Ho, K, a.n_cb, a.n_img, resident, band_h, min_band);
+  const long long tiles = static_cast<long long>(a.n_cb) * a.n_bands * a.n_img;
+  if (tiles > 0x7fffffffLL) return CONV2D_ESHAPE;
+  a.n_tiles = static_cast<int>(tiles);
+  auto go = [&]() {
+    kernel<<<a.n_tiles, kWarp, ring, stream>>>(a);
     return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
   };
   if constexpr (FSRC == FSRC_CONST) return with_const_filter(filt, K, KCfg<K>::KP, stream, dev, go);
@@ -237,7 +276,7 @@ int launch_split_v(const SingleGeom &g, const float *filt, float *out, cudaStrea
     }
     resident = v;
   }
-  a.n_bands = band_count(a.Ho, a.n_cb, a.n_img, resident, band_h, min_band);
+  a.n_bands = band_count(a.Ho, K, a.n_cb, a.n_img, resident, band_h, min_band);
   const long long tiles = static_cast<long long>(a.n_cb) * a.n_bands * a.n_img;
   if (tiles * G > 0x7fffffffLL) return CONV2D_ESHAPE;
   a.n_tiles = static_cast<int>(tiles);
@@ -342,6 +381,19 @@ int launch_single(const SingleGeom &g, const float *filt, float *out, cudaStream
     default: break;
   }
 #undef C2D_LS
+  // wide-lane kernel (conv2d_wide.cuh; variants 20-26)
+#define C2D_LW(FS, PFF, G) launch_wide_v<K, FS, PFF, G>(g, filt, out, stream, band_h, dev, min_band)
+  switch (tuning_variant()) {
+    case 20: if (constant_ok) return C2D_LW(FSRC_CONST, 1, 0); break;
+    case 21: if (constant_ok) return C2D_LW(FSRC_CONST, 1, 1); break;
+    case 22: if (constant_ok) return C2D_LW(FSRC_CONST, 1, 2); break;
+    case 23: if (constant_ok) return C2D_LW(FSRC_CONST, 4, 0); break;
+    case 24: if (constant_ok) return C2D_LW(FSRC_CONST, 4, 1); break;
+    case 25: if (constant_ok) return C2D_LW(FSRC_CONST, 4, 2); break;
+    case 26: return C2D_LW(FSRC_SMEM, 1, 0);
+    default: break;
+  }
+#undef C2D_LW
   // filter-row split (conv2d_split.cuh; variants 10-12)
 #define C2D_SP(GG, UU, PFF, RR, CLL) launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(g, filt, out, stream, band_h, dev, 1)
   const int v = tuning_variant();

@@ -39,23 +39,30 @@ def main():
     ap.add_argument("--variants", default="1,2,3,4")
     ap.add_argument("--band", type=int, default=0)
     ap.add_argument("--minband", type=int, default=0)
+    ap.add_argument("--batch", type=int, default=1, help="images per call (conv2d_single_batch when > 1)")
     a = ap.parse_args()
     _capi.debug_set_min_band(a.minband)
     for S in [int(v) for v in a.sizes.split(",")]:
-        x = synth.fill_torch(1, 1, (S, S), "img", device="cuda")
+        B = a.batch
+        x = synth.fill_torch(1, 1, (B, S, S), "img", device="cuda")
+
+        def call(x, f, out=None, band_h=0):
+            if B == 1:
+                return pkg.conv2d_single(x[0], f, out=None if out is None else out[0], band_h=band_h)[None]
+            return pkg.conv2d_single_batch(x, f, out=out)
         for K in [int(v) for v in a.ks.split(",")]:
             f = torch.from_numpy(synth.make_filter(1, K, "rand")[0, 0]).cuda()
             ref = None
             line = f"{S}^2 K={K:2d}:"
             for v in [int(t) for t in a.variants.split(",")]:
                 _capi.debug_set_variant(v)
-                y = pkg.conv2d_single(x, f, band_h=a.band)
+                y = call(x, f, band_h=a.band)
                 torch.cuda.synchronize()
                 if ref is None:
                     ref = y.clone()
                 same = torch.equal(y, ref)
-                ms = time_call(lambda: pkg.conv2d_single(x, f, out=y, band_h=a.band))
-                px = (S - K + 1) ** 2
+                ms = time_call(lambda: call(x, f, out=y, band_h=a.band))
+                px = (S - K + 1) ** 2 * B
                 line += f"  v{v} {px / ms / 1e6:7.1f} Gpx/s ({2 * px * K * K / ms / 1e9:5.1f} TF){'' if same else ' MISMATCH'}"
             _capi.debug_set_variant(0)
             print(line, flush=True)
