@@ -37,15 +37,18 @@ struct WideRow {
   float e[kWideV];  // lanes 0/1: the 8 columns at x0 + 256 + 8*lane (halo of lanes 31/30)
 };
 
-// a1: one input row of the tile. EDGE 0: 16B-aligned, every column of the span + halo inside the row:
-// 2 x LDG.128 own + 2 x LDG.128 halo (lanes >= 2 re-read lanes 0/1's halo: branch-free, same
-// sectors). EDGE 1: aligned rows, ragged right edge: quad addresses clamped to the row's last quad (a
-// valid output only reads inside quads; clamped garbage reaches only outputs >= Wo, never stored).
-// EDGE 2: misaligned rows: guarded scalar loads.
-template <int K, int EDGE>
-__device__ __forceinline__ void wide_load(WideRow &b, const float *__restrict__ rowp, int x0, int Wc, int lane) {
-  const int xa = x0 + kWideV * lane;
-  const int xe = x0 + kWideSpan + kWideV * (lane & 1);
+// a1: one input row of the tile. The warp is split into 32/SEG segments of SEG lanes (multi-channel:
+// one image per segment; single-channel: SEG = 32); segment lane sl owns columns x0 + 8*sl .. + 7 and
+// segment lanes 0/1 also hold the 16 columns right of the segment's span (x0 + 8*SEG + 8*sl).
+// EDGE 0: 16B-aligned, every column of the span + halo inside the row: 2 x LDG.128 own + 2 x LDG.128
+// halo (lanes >= 2 re-read lanes 0/1's halo: branch-free, same sectors). EDGE 1: aligned rows, ragged
+// right edge: quad addresses clamped to the row's last quad (a valid output only reads inside quads;
+// clamped garbage reaches only outputs >= Wo, never stored). EDGE 2: misaligned rows: guarded scalar
+// loads.
+template <int K, int EDGE, int SEG = kWarp>
+__device__ __forceinline__ void wide_load(WideRow &b, const float *__restrict__ rowp, int x0, int Wc, int sl) {
+  const int xa = x0 + kWideV * sl;
+  const int xe = x0 + kWideV * SEG + kWideV * (sl & 1);
   if constexpr (EDGE == 2) {
 #pragma unroll
     for (int t = 0; t < kWideV; ++t) b.a[t] = (xa + t < Wc) ? __ldg(rowp + xa + t) : 0.f;
@@ -58,16 +61,14 @@ __device__ __forceinline__ void wide_load(WideRow &b, const float *__restrict__ 
       const float4 v = ldg4(rowp + x);
       b.a[4 * h] = v.x; b.a[4 * h + 1] = v.y; b.a[4 * h + 2] = v.z; b.a[4 * h + 3] = v.w;
     }
-    if constexpr (K > 1) {
 #pragma unroll
-      for (int h = 0; h < 2; ++h) {
-        if (4 * h < K - 1) {  // static: only the halo quads the window uses
-          const int x = (EDGE == 1) ? min(xe + 4 * h, Wc - 4) : xe + 4 * h;
-          const float4 v = ldg4(rowp + x);
-          b.e[4 * h] = v.x; b.e[4 * h + 1] = v.y; b.e[4 * h + 2] = v.z; b.e[4 * h + 3] = v.w;
-        } else {
-          b.e[4 * h] = b.e[4 * h + 1] = b.e[4 * h + 2] = b.e[4 * h + 3] = 0.f;
-        }
+    for (int h = 0; h < 2; ++h) {
+      if (K > 1 && 4 * h < K - 1) {  // static: only the halo quads the window uses
+        const int x = (EDGE == 1) ? min(xe + 4 * h, Wc - 4) : xe + 4 * h;
+        const float4 v = ldg4(rowp + x);
+        b.e[4 * h] = v.x; b.e[4 * h + 1] = v.y; b.e[4 * h + 2] = v.z; b.e[4 * h + 3] = v.w;
+      } else {
+        b.e[4 * h] = b.e[4 * h + 1] = b.e[4 * h + 2] = b.e[4 * h + 3] = 0.f;
       }
     }
   }
@@ -75,16 +76,16 @@ __device__ __forceinline__ void wide_load(WideRow &b, const float *__restrict__ 
 
 // cp.async ring of wide rows: each lane copies its own 2 quads + its 2 halo quads global -> shared and
 // later reads back only what it wrote (no cross-lane synchronisation), NST stages per warp.
-template <int K, int NST>
+template <int K, int NST, int SEG = kWarp>
 struct WideRing {
   static constexpr unsigned kStageBytes = kWarp * 4 * 16;  // 4 quads per lane
   static constexpr unsigned kBytes = NST * kStageBytes;
   unsigned base;
-  int lane;
+  int lane, sl;
   __device__ __forceinline__ void issue(int stage, const float *__restrict__ rowp, int x0, int Wc, bool clamp) const {
     const unsigned sb = base + stage * kStageBytes + lane * 16;
-    const int xa = x0 + kWideV * lane;
-    const int xe = x0 + kWideSpan + kWideV * (lane & 1);
+    const int xa = x0 + kWideV * sl;
+    const int xe = x0 + kWideV * SEG + kWideV * (sl & 1);
 #pragma unroll
     for (int h = 0; h < 2; ++h) cp_async16(sb + h * kWarp * 16, rowp + (clamp ? min(xa + 4 * h, Wc - 4) : xa + 4 * h));
 #pragma unroll
@@ -107,18 +108,21 @@ struct WideRing {
   }
 };
 
-// a2: w[0..WN) = in[x0 + 8*lane .. + WN). Halo element m (m >= 8) of lane l is register m%8 of lane
-// l + m/8; a supplying lane s < m/8 serves a wrapped receiver (l = s - m/8 + 32) from its halo register.
-template <int K>
+// a2: w[0..WN) = in[x0 + 8*sl .. + WN). Halo element m (m >= 8) of segment lane sl is register m%8 of
+// segment lane sl + m/8; a supplying lane s < m/8 serves a wrapped receiver (sl = s - m/8 + SEG) from
+// its halo register. Shuffles stay inside the segment.
+template <int K, int SEG = kWarp>
 __device__ __forceinline__ void wide_window(const WideRow &b, float (&w)[WideCfg<K>::WN], int lane) {
+  const int sl = lane & (SEG - 1);
+  const int base = lane & ~(SEG - 1);
 #pragma unroll
   for (int t = 0; t < kWideV; ++t) w[t] = b.a[t];
 #pragma unroll
   for (int m = kWideV; m < WideCfg<K>::WN; ++m) {
     const int d = m / kWideV;  // source lane offset (static, 1 or 2)
     const int r = m % kWideV;  // source register (static)
-    const float sup = (lane < d) ? b.e[r] : b.a[r];
-    w[m] = __shfl_sync(kFull, sup, (lane + d) & (kWarp - 1));
+    const float sup = (sl < d) ? b.e[r] : b.a[r];
+    w[m] = __shfl_sync(kFull, sup, base | ((sl + d) & (SEG - 1)));
   }
 }
 
@@ -194,8 +198,8 @@ __device__ __forceinline__ void wide_store(float *__restrict__ orow, int x0, int
 }
 
 // One warp tile: 256 columns x output rows [ob, oe), input rows [ob, oe+K-1) streamed once (Alg. 2's
-// three cases as in single_tile). PF 1: the next row in flight in registers; PF >= 3 (power of two,
-// EDGE < 2): a PF-stage cp.async ring, PF-1 rows in flight. GUARDS as single_tile.
+// three cases as in single_tile). PF 1 / 2: the next one / two rows in flight in registers; PF >= 3
+// (power of two, EDGE < 2): a PF-stage cp.async ring, PF-1 rows in flight. GUARDS as single_tile.
 template <int K, int FSRC, int PF, int GUARDS, int EDGE, bool HALO>
 __device__ __forceinline__ void wide_tile(const SingleArgs &a, const float *__restrict__ inb, float *__restrict__ outb,
                                           const FilterSrc<K, FSRC> &fs, int x0, int ob, int oe, int lane,
@@ -213,13 +217,18 @@ __device__ __forceinline__ void wide_tile(const SingleArgs &a, const float *__re
   WideRing<K, (NST > 1 ? NST : 2)> ring;
   ring.base = ring_base;
   ring.lane = lane;
-  WideRow n1;
+  ring.sl = lane;
+  WideRow n1, n2;  // register path: rows r+1 (and r+2 when PF == 2) in flight
   if constexpr (NST > 1) {
 #pragma unroll
     for (int st = 0; st < NST - 1; ++st) ring.issue(st, in_row<HALO>(a, inb, min(ob + st, rlast)), x0, a.Wc, EDGE == 1);
   } else {
     wide_load<K, EDGE>(n1, in_row<HALO>(a, inb, ob), x0, a.Wc, lane);
+    if constexpr (PF == 2) wide_load<K, EDGE>(n2, in_row<HALO>(a, inb, min(ob + 1, rlast)), x0, a.Wc, lane);
   }
+  // returns row r and issues the fetch of row r + depth (index clamped). PF == 2: the copy n1 = n2 reads
+  // a row fetched one full iteration earlier, so it never waits on the load (PF == 1's cur = n1 copy
+  // stalls on a load issued late in the previous iteration -- ncu long_scoreboard at that MOV).
   auto next_row = [&](int r) {
     WideRow cur;
     if constexpr (NST > 1) {
@@ -227,6 +236,10 @@ __device__ __forceinline__ void wide_tile(const SingleArgs &a, const float *__re
       const int k = r - ob;
       ring.read(k & (NST - 1), cur);
       ring.issue((k + NST - 1) & (NST - 1), in_row<HALO>(a, inb, min(r + NST - 1, rlast)), x0, a.Wc, EDGE == 1);
+    } else if constexpr (PF == 2) {
+      cur = n1;
+      n1 = n2;
+      wide_load<K, EDGE>(n2, in_row<HALO>(a, inb, min(r + 2, rlast)), x0, a.Wc, lane);
     } else {
       cur = n1;
       wide_load<K, EDGE>(n1, in_row<HALO>(a, inb, min(r + 1, rlast)), x0, a.Wc, lane);

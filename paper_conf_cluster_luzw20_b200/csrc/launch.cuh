@@ -378,6 +378,10 @@ int launch_single(const SingleGeom &g, const float *filt, float *out, cudaStream
     case 9: if (constant_ok) return C2D_LS(1, FSRC_CONST, 4, 2); break;
     case 13: if constexpr (K >= 5 && K <= 9) { if (constant_ok) return C2D_LS(2, FSRC_CONST, 4, 2); } break;
     case 15: if constexpr (K >= 10) { if (constant_ok) return C2D_LS(1, FSRC_CONST, 4, 1); } break;
+    case 16: if (constant_ok) return C2D_LS(1, FSRC_CONST, 2, 1); break;
+    case 17: if (constant_ok) return C2D_LS(1, FSRC_CONST, 2, 0); break;
+    case 18: if (constant_ok) return C2D_LS(2, FSRC_CONST, 2, 0); break;
+    case 19: if (constant_ok) return C2D_LS(1, FSRC_CONST, 2, 2); break;
     default: break;
   }
 #undef C2D_LS
@@ -391,6 +395,9 @@ int launch_single(const SingleGeom &g, const float *filt, float *out, cudaStream
     case 24: if (constant_ok) return C2D_LW(FSRC_CONST, 4, 1); break;
     case 25: if (constant_ok) return C2D_LW(FSRC_CONST, 4, 2); break;
     case 26: return C2D_LW(FSRC_SMEM, 1, 0);
+    case 27: if (constant_ok) return C2D_LW(FSRC_CONST, 2, 0); break;
+    case 28: if (constant_ok) return C2D_LW(FSRC_CONST, 2, 2); break;
+    case 29: return C2D_LW(FSRC_SMEM, 2, 0);
     default: break;
   }
 #undef C2D_LW
