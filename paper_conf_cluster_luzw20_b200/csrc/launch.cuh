@@ -15,6 +15,7 @@
 #include "conv2d_multi.cuh"
 #include "conv2d_split.cuh"
 #include "conv2d_wide.cuh"
+#include "conv2d_mwide.cuh"
 
 namespace {
 
@@ -297,6 +298,7 @@ template <int K, bool HALO>
 int launch_single_default(const SingleGeom &g, const float *filt, float *out, cudaStream_t stream, int band_h,
                           const DevInfo &dev, int min_band, bool constant_ok) {
 #define C2D_LS(UU, FS, PFF, G) launch_single_v<K, UU, FS, PFF, G, HALO>(g, filt, out, stream, band_h, dev, min_band)
+#define C2D_LW(FS, PFF, G) launch_wide_v<K, FS, PFF, G, HALO>(g, filt, out, stream, band_h, dev, min_band)
 #define C2D_SP(GG, UU, PFF, RR, CLL) launch_split_v<K, GG, UU, PFF, RR, 1, CLL>(g, filt, out, stream, band_h, dev, 1)
   const int W = g.W;
   const bool force_smem = band_h == kBandSmemFilter;
@@ -310,34 +312,42 @@ int launch_single_default(const SingleGeom &g, const float *filt, float *out, cu
     if (constant_ok && W <= 1024 && !no_split) return C2D_SP(2, 1, 4, 4, 1);
   }
 #undef C2D_SP
-  // Tuned on B200 (tools/variants.py sweeps):
-  //   K <= 5        two 128-column chunks per warp; row fetch from a 4-stage cp.async ring, except
-  //                 K <= 3 on wide images (one register row in flight is enough when HBM-bound);
-  //   K = 6..9      wide images (W >= 8192): two chunks + ring; narrower: one chunk + ring with
-  //                 Alg. 2 case-1/3 guards (short bands);
+  // Tuned on B200 (tools/variants.py sweeps, profiles/r02e_variants*.txt):
+  //   K <= 3        the wide-lane kernel (8 contiguous columns per lane): constant-slot filter on wide
+  //                 images, per-CTA shared-memory filter below (no slot staging: 4096^2 511 vs 444 Gpx/s);
+  //   K = 4, 5      images up to 2048 wide: wide lanes + shared-memory filter; wider: two 128-column
+  //                 chunks per warp with a 4-stage cp.async row ring;
+  //   K = 6..9      W >= 8192: wide lanes, both Alg. 2 edge cases guarded (8192^2 K=9 325 vs 307 Gpx/s,
+  //                 K=7 457 vs 449; batches of 8: 340 vs 335, 503 vs 491); narrower: one or two chunks +
+  //                 ring + guards;
   //   K = 10, 11    one chunk + ring + guards;
-  //   K >= 12       one chunk, register row fetch, guarded prologue on wide images (tall bands),
-  //                 guarded prologue + epilogue on narrow ones.
+  //   K >= 12       one chunk (the wide kernel's 32 KB loop body overflows the instruction cache at
+  //                 K >= 11: ncu no_instructions 20% at K=15), register row fetch, guarded prologue on
+  //                 wide images, guarded prologue + epilogue on narrow ones.
   // Small images with K < 11 are latency-bound (a few microseconds): the per-CTA shared-memory filter
   // skips the constant-slot staging (a stream-ordered copy plus two event operations, ~3 us of host
   // and device time per call, tools/host_overhead.py). Same summation order, same bits.
-  // (tools/small_sizes2.py, back-to-back calls: 1024^2 K=3 12.1 -> 8.0 us, K=5 12.0 -> 10.3 us)
   const long long px = static_cast<long long>(g.H) * W * g.N;
   const bool small = px <= 512LL * 512 || (K <= 5 && px <= 1024LL * 1024);
+  if constexpr (K <= 3) {
+    if (constant_ok && !force_smem && W >= 8192) return C2D_LW(FSRC_CONST, 1, 2);
+    return C2D_LW(FSRC_SMEM, 1, 0);
+  }
+  if constexpr (K <= 5) {
+    if (!constant_ok || force_smem || W <= 2048) return C2D_LW(FSRC_SMEM, 1, 0);
+  }
   if (!constant_ok || force_smem || (K < 11 && small)) {
     if constexpr (K <= 7) return C2D_LS(2, FSRC_SMEM, 1, 0);
     else return C2D_LS(1, FSRC_SMEM, 1, 0);
   }
   if constexpr (K <= 5) {
-    if (K <= 3 && W > 1024) return C2D_LS(2, FSRC_CONST, 1, 0);
     return C2D_LS(2, FSRC_CONST, 4, 0);
   } else if constexpr (K <= 7) {
-    // K = 6, 7: two chunks + ring with both Alg. 2 edge cases guarded on wide images
-    // (tools/split_sweep.py variant 14: 8192^2 K=7 445 -> 458 Gpx/s, 4096^2 333 -> 348)
+    if (W >= 8192) return C2D_LW(FSRC_CONST, 1, 2);
     if (W >= 4096) return C2D_LS(2, FSRC_CONST, 4, 2);
     return C2D_LS(1, FSRC_CONST, 4, 2);
   } else if constexpr (K <= 9) {
-    if (W >= 8192) return C2D_LS(2, FSRC_CONST, 4, 0);
+    if (W >= 8192) return C2D_LW(FSRC_CONST, 1, 2);
     return C2D_LS(1, FSRC_CONST, 4, 2);
   } else if constexpr (K <= 11) {
     return C2D_LS(1, FSRC_CONST, 4, 2);
@@ -349,6 +359,7 @@ int launch_single_default(const SingleGeom &g, const float *filt, float *out, cu
     return C2D_LS(1, FSRC_CONST, 1, 2);
   }
 #undef C2D_LS
+#undef C2D_LW
 }
 
 template <int K>
@@ -545,6 +556,82 @@ int launch_multi2_v(const float *in, int N, int C, int H, int W, const float *fi
   return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
 }
 
+// Multi-channel band choice shared by the multi kernels: K >= 5 one full wave of resident warps (the
+// K-1 prologue rows of extra bands cost more than the wave quantisation they remove --
+// tools/multi_band_sweep.py: Table I CONV3/CONV5, configs[3]); K <= 4 the wave-quantisation cost model
+// b* = argmin waves(b) * (ceil(Ho / b) + K - 1) (one band per tile whenever the (image group, F-block,
+// column-block) groups alone exceed a wave had left Table I CONV11 at 1.15 waves: 946 -> 570 us).
+// Returns n_bands padded so that the 4 warps of a CTA share (group, F-block); sets band_h.
+template <int K>
+int multi_bands(int Ho, int n_cb, long long groups, long long resident_ctas, int &band_h) {
+  if (band_h <= 0 && K >= 5) {
+    const long long resident_warps = resident_ctas * kCtaWarps;
+    long long bands = resident_warps / (groups * n_cb);
+    if (bands < 1) bands = 1;
+    band_h = ceil_div(Ho, bands);
+  } else if (band_h <= 0) {
+    long long best_b = 1;
+    double best = 1e300;
+    const int bmax = Ho < 512 ? Ho : 512;
+    for (int b = 1; b <= bmax; ++b) {
+      const int h = ceil_div(Ho, b);
+      const int nb = ceil_div(Ho, h);  // bands actually used with height h
+      long long nbp = nb;
+      while ((static_cast<long long>(n_cb) * nbp) % kCtaWarps) ++nbp;
+      const long long ctas = groups * n_cb * nbp / kCtaWarps;
+      const long long waves = (ctas + resident_ctas - 1) / resident_ctas;
+      const double cost = static_cast<double>(waves) * (h + K - 1) * (1.0 + 1e-3 * (nbp - nb));
+      if (cost < best - 1e-9) {
+        best = cost;
+        best_b = nb;
+      }
+    }
+    band_h = ceil_div(Ho, best_b);
+  }
+  if (band_h > Ho) band_h = Ho;
+  int n_bands = ceil_div(Ho, band_h);
+  while ((static_cast<long long>(n_cb) * n_bands) % kCtaWarps) ++n_bands;
+  return n_bands;
+}
+
+// Wide-lane multi-channel kernel (conv2d_mwide.cuh): FB filters per warp, SEG-lane segments of 8*SEG
+// columns, PF (row, channel) entries in flight in registers.
+template <int K, int FB, int SEG, int GUARDS, int PF, int MINB>
+int launch_mwide_v(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
+                   cudaStream_t stream, int band_h, const DevInfo &dev) {
+  constexpr int KP = KCfg<K>::KP;
+  constexpr int SEGS = kWarp / SEG;
+  auto kernel = k_conv2d_mwide<K, FB, SEG, GUARDS, PF, MINB>;
+  static OccCache occ_cache;
+  static SmemOptIn smem_flag;
+  const size_t smem = static_cast<size_t>(C) * K * FB * KP * sizeof(float);
+  if (int e = ensure_smem(kernel, smem, dev, smem_flag)) return e;
+  Multi2Args a;
+  a.in = in;
+  a.filt = filt;
+  a.out = out;
+  a.N = N;
+  a.C = C;
+  a.H = H;
+  a.W = W;
+  a.F = F;
+  a.Ho = H - K + 1;
+  a.Wo = W - K + 1;
+  a.n_cb = ceil_div(a.Wo, kWideV * SEG);
+  a.n_fb = ceil_div(F, FB);
+  a.n_groups = ceil_div(N, SEGS);
+  a.aligned = (aligned16(in) && (W % 4 == 0)) ? 1 : 0;
+  const long long resident_ctas =
+      static_cast<long long>(cta_occupancy(kernel, smem, occ_cache, kCtaWarps * kWarp)) * dev.num_sms;
+  a.n_bands = multi_bands<K>(a.Ho, a.n_cb, static_cast<long long>(a.n_groups) * a.n_fb, resident_ctas, band_h);
+  a.band_h = band_h;
+  a.n_tiles = static_cast<long long>(a.n_groups) * a.n_fb * a.n_bands * a.n_cb;
+  const long long blocks = (a.n_tiles + kCtaWarps - 1) / kCtaWarps;
+  if (blocks > 0x7fffffffLL) return CONV2D_ESHAPE;
+  kernel<<<static_cast<unsigned>(blocks), kCtaWarps * kWarp, smem, stream>>>(a);
+  return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
+}
+
 // fraction of a segment-row's lanes doing valid columns
 inline double lane_use(int Wo, int span) { return double(Wo) / (double(ceil_div(Wo, span)) * span); }
 
@@ -584,6 +671,24 @@ int launch_multi(const float *in, int N, int C, int H, int W, const float *filt,
   if (mv == 4) return C2D_LM(FBH, 16);
   if (mv == 7) return (K > 3) ? C2D_LM(FBH, 8) : C2D_LM(FB, 8);
 #undef C2D_LM2
+  {
+    // wide-lane kernel (conv2d_mwide.cuh), variants 60-69: SEG x {PF 1, 2}
+    constexpr int FBW = (K <= 3) ? 4 : (K <= 8 ? 2 : 1);
+#define C2D_LMW(SEGG, PFF) \
+  launch_mwide_v<K, FBW, SEGG, GUARDS, PFF, 2>(in, N, C, H, W, filt, F, out, stream, band_h, dev)
+    switch (mv) {
+      case 60: return C2D_LMW(32, 1);
+      case 61: return C2D_LMW(32, 2);
+      case 62: return C2D_LMW(16, 1);
+      case 63: return C2D_LMW(16, 2);
+      case 64: return C2D_LMW(8, 1);
+      case 65: return C2D_LMW(8, 2);
+      case 66: return C2D_LMW(4, 1);
+      case 67: return C2D_LMW(4, 2);
+      default: break;
+    }
+#undef C2D_LMW
+  }
 #endif
   // Tuned on B200 (tools/multi_variants.py): 16-lane segments (two images per warp) unless they waste
   // clearly more lanes than whole-warp rows -- more column blocks take the vector fast path and the

@@ -25,6 +25,9 @@ SHAPES = {  # name: (N, C, H, W, F, K)
     "TableI CONV9 C3": (128, 3, 56, 56, 256, 3),
     "TableI CONV11 C1": (128, 1, 224, 224, 64, 3),
 }
+TABLE1 = [("CONV1", 28, 128, 3), ("CONV2", 56, 64, 3), ("CONV3", 12, 64, 5), ("CONV4", 14, 16, 5),
+          ("CONV5", 24, 256, 5), ("CONV6", 24, 64, 5), ("CONV7", 28, 16, 5), ("CONV8", 28, 512, 3),
+          ("CONV9", 56, 256, 3), ("CONV10", 112, 128, 3), ("CONV11", 224, 64, 3)]
 
 
 def time_call(fn, n=10):
@@ -46,8 +49,15 @@ def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("--variants", default="0,1,2,3,4,9")
     ap.add_argument("--only", default="")
+    ap.add_argument("--table1", action="store_true", help="all 22 Table I layers (C in {1, 3}) + the two configs")
     a = ap.parse_args()
-    for name, (N, C, H, W, F, K) in SHAPES.items():
+    shapes = dict(SHAPES)
+    if a.table1:
+        shapes = {k: v for k, v in SHAPES.items() if k.startswith("config")}
+        for C in (1, 3):
+            for nm, S, F, K in TABLE1:
+                shapes[f"TableI {nm} C{C}"] = (128, C, S, S, F, K)
+    for name, (N, C, H, W, F, K) in shapes.items():
         if a.only and a.only not in name:
             continue
         x = synth.fill_torch(1, 1, (N, C, H, W), "img", device="cuda")
