@@ -44,6 +44,7 @@ def lib():
         L.oracle_num_threads.restype = ctypes.c_int
         L.oracle_conv2d_single_rows.argtypes = [_P, _I, _I, _P, _I, _I, _I, _P, _P, _P]
         L.oracle_conv2d_single.argtypes = [_P, _I, _I, _P, _I, _P, _P, _P]
+        L.oracle_conv2d_single_rect.argtypes = [_P, _I, _I, _P, _I, _I, _P, _P, _P]
         L.oracle_conv2d_single_points.argtypes = [_P, _I, _I, _P, _I, _P, _P, _I, _P, _P]
         L.oracle_conv2d_multi_images.argtypes = [_P, _I, _I, _I, _I, _P, _I, _I, _I, _I, _P, _P, _P]
         L.oracle_conv2d_multi.argtypes = [_P, _I, _I, _I, _I, _P, _I, _I, _P, _P, _P]
@@ -84,6 +85,22 @@ def conv2d_single(image, filt, want_bound=True, want_f64=False, rows=None):
     y0, y1 = (0, Ho) if rows is None else rows
     lib().oracle_conv2d_single_rows(_ptr(image), H, W, _ptr(filt), K, y0, y1, _ptr(out), _ptr(bound),
                                     _ptr(out64))
+    return out, bound, out64
+
+
+def conv2d_single_rect(image, filt, want_bound=True, want_f64=False):
+    """Plain-definition valid cross-correlation with a rectangular FH x FW filter (conv2d_oracle.c
+    oracle_conv2d_single_rect). Returns (out fp32, bound f64 or None, out64 or None)."""
+    image = _f32(image)
+    filt = _f32(filt)
+    H, W = image.shape
+    FH, FW = filt.shape
+    assert H >= FH and W >= FW
+    Ho, Wo = H - FH + 1, W - FW + 1
+    out = np.empty((Ho, Wo), np.float32)
+    bound = np.empty((Ho, Wo), np.float64) if want_bound else None
+    out64 = np.empty((Ho, Wo), np.float64) if want_f64 else None
+    lib().oracle_conv2d_single_rect(_ptr(image), H, W, _ptr(filt), FH, FW, _ptr(out), _ptr(bound), _ptr(out64))
     return out, bound, out64
 
 

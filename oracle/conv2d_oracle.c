@@ -103,6 +103,36 @@ void oracle_conv2d_single_points(const float *in, int64_t H, int64_t W, const fl
     }
 }
 
+/*
+ * Rectangular FH x FW filters (Table I lists filters as "FH x FW", P:338 --
+ * every entry there is square, the variant is the image-library generalisation):
+ *     out[y][x] = fl32( sum_{i<FH} sum_{j<FW} (double)in[y+i][x+j] * (double)f[i][j] )
+ * in: H*W row-major. f: FH*FW row-major. out / bound / out64: (H-FH+1)*(W-FW+1) row-major (each may be
+ * NULL). Same order and single rounding as the square definition above.
+ */
+void oracle_conv2d_single_rect(const float *in, int64_t H, int64_t W, const float *f, int64_t FH, int64_t FW,
+                               float *out, double *bound, double *out64)
+{
+    const int64_t Ho = H - FH + 1, Wo = W - FW + 1;
+#pragma omp parallel for schedule(dynamic, 1)
+    for (int64_t y = 0; y < Ho; ++y) {
+        for (int64_t x = 0; x < Wo; ++x) {
+            double acc = 0.0, b = 0.0;
+            for (int64_t i = 0; i < FH; ++i) {
+                for (int64_t j = 0; j < FW; ++j) {
+                    double p = (double)in[(y + i) * W + (x + j)] * (double)f[i * FW + j];
+                    acc += p;
+                    b += fabs(p);
+                }
+            }
+            const int64_t o = y * Wo + x;
+            if (out) out[o] = (float)acc;
+            if (bound) bound[o] = b;
+            if (out64) out64[o] = acc;
+        }
+    }
+}
+
 /* One output element of the multi-channel definition. */
 static void multi_point(const float *in, int64_t C, int64_t H, int64_t W, const float *w, int64_t K,
                         int64_t n, int64_t f, int64_t y, int64_t x, double *acc_out, double *bound_out)

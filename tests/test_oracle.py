@@ -314,3 +314,78 @@ def test_flip_impulse_gives_filter_upright(K):
     exp = np.zeros_like(y)
     exp[r0 - K + 1:r0 + 1, c0 - K + 1:c0 + 1] = f
     assert np.array_equal(y, exp)
+
+
+# --------------------------------------------------------------------------------------------
+# Rectangular FH x FW filters (Table I's "FH x FW" columns)
+# --------------------------------------------------------------------------------------------
+RECT_SHAPES = [(1, 5), (5, 1), (3, 7), (7, 3), (2, 15), (15, 2), (4, 9), (13, 6)]
+
+
+def test_rect_matches_scipy_correlate2d_bruteforce():
+    """Textbook routine: scipy.signal.correlate2d(mode='valid') in float64 on tiny shapes."""
+    import scipy.signal
+
+    rng = np.random.default_rng(7)
+    for FH, FW in RECT_SHAPES:
+        for dh, dw in [(0, 0), (1, 3), (6, 2)]:
+            x = rng.standard_normal((FH + dh, FW + dw)).astype(np.float32)
+            f = rng.standard_normal((FH, FW)).astype(np.float32)
+            y, bound, y64 = oracle.conv2d_single_rect(x, f, want_f64=True)
+            ref = scipy.signal.correlate2d(x.astype(np.float64), f.astype(np.float64), mode="valid")
+            assert y.shape == ref.shape == (dh + 1, dw + 1)
+            assert np.all(np.abs(y64 - ref) <= 1e-12 * bound)
+            assert np.array_equal(y, ref.astype(np.float32))
+
+
+def test_rect_delta_filter_is_shift():
+    """Closed form: a delta at (i0, j0) of an FH x FW filter shifts the image by (i0, j0)."""
+    x = synth.fill_np(3, synth.TAG_INPUT, (30, 41), "sym")
+    for FH, FW in RECT_SHAPES:
+        for i0, j0 in [(0, 0), (FH - 1, FW - 1), (FH // 2, FW - 1)]:
+            f = np.zeros((FH, FW), np.float32)
+            f[i0, j0] = 1.0
+            y, _, _ = oracle.conv2d_single_rect(x, f)
+            assert np.array_equal(y, x[i0:i0 + 30 - FH + 1, j0:j0 + 41 - FW + 1])
+
+
+def test_rect_box_filter_matches_summed_area_table():
+    """Closed form: an all-ones FH x FW filter on integer data sums the FH x FW window (prefix sums)."""
+    x = synth.fill_np(5, synth.TAG_INPUT, (40, 50), "int").astype(np.int64)
+    S = np.zeros((41, 51), np.int64)
+    S[1:, 1:] = x.cumsum(0).cumsum(1)
+    for FH, FW in RECT_SHAPES:
+        y, _, _ = oracle.conv2d_single_rect(x.astype(np.float32), np.ones((FH, FW), np.float32))
+        ref = S[FH:, FW:] - S[:-FH, FW:] - S[FH:, :-FW] + S[:-FH, :-FW]
+        assert np.array_equal(y, ref.astype(np.float32))
+
+
+def test_rect_square_reduces_to_single_and_transpose_swaps_shape():
+    """Invariants: FH == FW is the square definition; correlating the transposed image with the
+    transposed filter gives the transposed output (catches an FH/FW or i/j swap)."""
+    x = synth.fill_np(9, synth.TAG_INPUT, (33, 47), "img")
+    for K in (1, 4, 9):
+        f = synth.make_filter(9, K, "rand")[0, 0]
+        assert np.array_equal(oracle.conv2d_single_rect(x, f)[0], oracle.conv2d_single(x, f)[0])
+    rng = np.random.default_rng(3)
+    for FH, FW in RECT_SHAPES:
+        f = rng.standard_normal((FH, FW)).astype(np.float32)
+        y, _, _ = oracle.conv2d_single_rect(x, f)
+        yt, _, _ = oracle.conv2d_single_rect(np.ascontiguousarray(x.T), np.ascontiguousarray(f.T))
+        assert yt.shape == y.T.shape
+        assert np.allclose(yt, y.T, rtol=1e-6, atol=1e-6)
+
+
+def test_rect_separable_filter():
+    """Closed form: f = u v^T (FH x 1 times 1 x FW) is a column correlation by u after a row
+    correlation by v."""
+    x = synth.fill_np(11, synth.TAG_INPUT, (25, 31), "sym")
+    rng = np.random.default_rng(11)
+    for FH, FW in RECT_SHAPES:
+        u = rng.integers(-3, 4, (FH, 1)).astype(np.float32)
+        v = rng.integers(-3, 4, (1, FW)).astype(np.float32)
+        xi = np.round(x * 8).astype(np.float32)  # integers: every order exact
+        rows, _, _ = oracle.conv2d_single_rect(xi, v)
+        both, _, _ = oracle.conv2d_single_rect(rows, u)
+        direct, _, _ = oracle.conv2d_single_rect(xi, u @ v)
+        assert np.array_equal(both, direct)
