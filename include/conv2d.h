@@ -91,6 +91,19 @@ int conv2d_single_batch(const float *in, int N, int H, int W, const float *filt,
                         void *stream);
 
 /*
+ * Rectangular FH x FW filters (Table I's "FH x FW" filter columns): the same
+ * valid, stride-1 cross-correlation with a non-square filter,
+ *   filt : FH*FW floats, row-major:      filt[i*FW + j]
+ *   out  : (H-FH+1)*(W-FW+1) floats:     out[y*(W-FW+1) + x] = sum_{i<FH} sum_{j<FW} in[(y+i)*W + x+j] * filt[i*FW + j]
+ * 1 <= FH, FW <= 15 (CONV2D_EK above; CONV2D_ESHAPE for FH or FW < 1, H < FH, W < FW). FH == FW is
+ * conv2d_single. The kernel is the wide-lane column + row reuse kernel with an FH-slot ring and an
+ * FW-wide window (both compile-time), the filter staged per CTA in shared memory; each output sums in
+ * filter-row, filter-column order (exact on integer data). Same layouts, ownership, stream semantics.
+ */
+int conv2d_single_rect(const float *in, int H, int W, const float *filt, int FH, int FW, float *out,
+                       void *stream);
+
+/*
  * Same as conv2d_single / conv2d_multi with an explicit output-row band height per warp
  * (band_h <= 0: the library's choice). For tuning sweeps and tests of the band / halo logic; the
  * result is bitwise identical for every band_h (each output's summation order does not depend on
@@ -192,7 +205,7 @@ int conv2d_release_scratch(void);
 /* Human-readable text for a return code (static storage, never NULL). */
 const char *conv2d_strerror(int code);
 
-/* ABI version (major*100 + minor): 102 = conv2d_single_batch. */
+/* ABI version (major*100 + minor): 102 = conv2d_single_batch, 103 = conv2d_single_rect. */
 int conv2d_version(void);
 
 #ifdef __cplusplus

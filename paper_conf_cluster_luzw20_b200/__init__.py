@@ -10,8 +10,8 @@ The product is libconv2d.so (C ABI, include/conv2d.h). This package is its thin 
 """
 from . import _capi
 from .api import (conv2d_multi, conv2d_multi_host, conv2d_multi_tc, conv2d_single, conv2d_single_batch,
-                  conv2d_single_direct, conv2d_single_halo, conv2d_single_host, conv2d_single_pad)
+                  conv2d_single_direct, conv2d_single_rect, conv2d_single_halo, conv2d_single_host, conv2d_single_pad)
 
 __all__ = ["_capi", "conv2d_multi", "conv2d_multi_host", "conv2d_multi_tc", "conv2d_single",
-           "conv2d_single_batch", "conv2d_single_direct", "conv2d_single_halo", "conv2d_single_host",
+           "conv2d_single_batch", "conv2d_single_direct", "conv2d_single_rect", "conv2d_single_halo", "conv2d_single_host",
            "conv2d_single_pad"]

@@ -13,7 +13,7 @@ LIB_PATH = os.path.join(_PKG, "libconv2d.so")
 TUNE_LIB_PATH = os.path.join(_PKG, "libconv2d_tune.so")
 
 # every symbol include/conv2d.h declares
-EXPORTS = ("conv2d_single", "conv2d_single_batch", "conv2d_multi", "conv2d_single_ex", "conv2d_multi_ex", "conv2d_single_halo",
+EXPORTS = ("conv2d_single", "conv2d_single_batch", "conv2d_single_rect", "conv2d_multi", "conv2d_single_ex", "conv2d_multi_ex", "conv2d_single_halo",
            "conv2d_single_pad",
            "conv2d_single_direct",
            "conv2d_single_host", "conv2d_multi_tc", "conv2d_release_scratch", "conv2d_strerror", "conv2d_version")
@@ -46,6 +46,7 @@ def _declare(L):
     L.conv2d_single.argtypes = [P, I, I, P, I, P, P]
     L.conv2d_single_ex.argtypes = [P, I, I, P, I, P, P, I]
     L.conv2d_single_batch.argtypes = [P, I, I, I, P, I, P, P]
+    L.conv2d_single_rect.argtypes = [P, I, I, P, I, I, P, P]
     L.conv2d_single_halo.argtypes = [P, I, I, P, I, P, I, P, P]
     L.conv2d_single_pad.argtypes = [P, I, I, P, I, I, P, P]
     L.conv2d_single_direct.argtypes = [P, I, I, P, I, P, P]
@@ -151,6 +152,10 @@ def conv2d_single(in_ptr, H, W, filt_ptr, K, out_ptr, stream=0) -> int:
 
 def conv2d_single_batch(in_ptr, N, H, W, filt_ptr, K, out_ptr, stream=0) -> int:
     return lib().conv2d_single_batch(in_ptr, N, H, W, filt_ptr, K, out_ptr, stream)
+
+
+def conv2d_single_rect(in_ptr, H, W, filt_ptr, FH, FW, out_ptr, stream=0) -> int:
+    return lib().conv2d_single_rect(in_ptr, H, W, filt_ptr, FH, FW, out_ptr, stream)
 
 
 def conv2d_single_ex(in_ptr, H, W, filt_ptr, K, out_ptr, stream=0, band_h=0) -> int:

@@ -118,6 +118,25 @@ def conv2d_single_batch(x: torch.Tensor, f: torch.Tensor, out: torch.Tensor | No
     return out
 
 
+def conv2d_single_rect(x: torch.Tensor, f: torch.Tensor, out: torch.Tensor | None = None,
+                       stream=None) -> torch.Tensor:
+    """Valid cross-correlation with a rectangular filter f (FH, FW) -> (H-FH+1, W-FW+1)
+    (include/conv2d.h conv2d_single_rect)."""
+    _check_dev(x, "x")
+    _check_dev(f, "f")
+    if x.dim() != 2 or f.dim() != 2:
+        raise ValueError("x must be (H, W) and f (FH, FW)")
+    _check_same_device(x, f)
+    H, W = x.shape
+    FH, FW = f.shape
+    out = _out_for(out, (max(H - FH + 1, 0), max(W - FW + 1, 0)), x)
+    dev = x.device.index
+    with _on_device(dev):
+        _capi.check(_capi.conv2d_single_rect(x.data_ptr(), H, W, f.data_ptr(), FH, FW, out.data_ptr(),
+                                             _stream_handle(stream, dev)))
+    return out
+
+
 def conv2d_single_halo(x: torch.Tensor, halo: torch.Tensor, f: torch.Tensor, out: torch.Tensor | None = None,
                        stream=None) -> torch.Tensor:
     """conv2d_single of the rows of x followed by the rows of halo (same width), without concatenating

@@ -54,6 +54,10 @@ constexpr int kBandSmemFilter = -3;
 template <int K>
 int single_entry(const float *in, int N, int H, int W, const float *filt, float *out, cudaStream_t stream,
                  int band_h, const DevInfo &dev, const float *in2, int H1, long long P, int Po);
+// Rectangular KH x KW filters (KH a template parameter: one translation unit per KH, inst_rect_khNN.cu)
+template <int KH>
+int rect_entry(const float *in, int H, int W, const float *filt, int KW, float *out, cudaStream_t stream,
+               const DevInfo &dev);
 template <int K>
 int multi_entry(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
                 cudaStream_t stream, int band_h, const DevInfo &dev);

@@ -162,6 +162,26 @@ int conv2d_single_batch(const float *in, int N, int H, int W, const float *filt,
   return single_batch_impl(in, N, H, W, filt, K, out, stream, 0);
 }
 
+int conv2d_single_rect(const float *in, int H, int W, const float *filt, int FH, int FW, float *out,
+                       void *stream) {
+  if (!in || !filt || !out) return CONV2D_ENULL;
+  if (FH < 1 || FW < 1) return CONV2D_ESHAPE;
+  if (FH > CONV2D_MAX_K || FW > CONV2D_MAX_K) return CONV2D_EK;
+  if (H < FH || W < FW) return CONV2D_ESHAPE;
+  if (!aligned4(in) || !aligned4(filt) || !aligned4(out)) return CONV2D_EALIGN;
+  const size_t in_b = static_cast<size_t>(H) * W * sizeof(float);
+  const size_t out_b = static_cast<size_t>(H - FH + 1) * (W - FW + 1) * sizeof(float);
+  const size_t f_b = static_cast<size_t>(FH) * FW * sizeof(float);
+  if (overlap(in, in_b, out, out_b) || overlap(filt, f_b, out, out_b)) return CONV2D_EOVERLAP;
+  if (FH == FW) return single_batch_impl(in, 1, H, W, filt, FH, out, stream, 0);  // square: conv2d_single
+  DevInfo dev;
+  if (current_device_info(&dev)) return CONV2D_ECUDA;
+  cudaStream_t s = static_cast<cudaStream_t>(stream);
+#define C2D_CALL_RECT(KK) rect_entry<KK>(in, H, W, filt, FW, out, s, dev)
+  C2D_K_SWITCH(FH, C2D_CALL_RECT)
+#undef C2D_CALL_RECT
+}
+
 int conv2d_single_halo(const float *in, int H, int W, const float *halo, int halo_rows, const float *filt, int K,
                        float *out, void *stream) {
   if (halo_rows < 0) return CONV2D_ESHAPE;
@@ -250,7 +270,7 @@ const char *conv2d_strerror(int code) {
   }
 }
 
-int conv2d_version(void) { return 102; }
+int conv2d_version(void) { return 103; }
 
 int conv2d_release_scratch(void) { return scratch_trim() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA; }
 

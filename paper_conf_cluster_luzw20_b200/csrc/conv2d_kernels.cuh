@@ -609,7 +609,9 @@ __device__ __forceinline__ void multi_tile(const MultiArgs &a, const float *__re
       for (int fb = 0; fb < FB; ++fb) {
         if (f0 + fb < a.F) {
           float *orow = a.out + ((static_cast<size_t>(n) * a.F + f0 + fb) * a.Ho + o) * a.Wo;
-          const float(&ov)[1][4] = *reinterpret_cast<const float(*)[1][4]>(&acc[0][fb][0]);
+          float ov[1][4];
+#pragma unroll
+          for (int v = 0; v < 4; ++v) ov[0][v] = acc[0][fb][v];
           store_row<1, SAFE>(orow, x0, a.Wo, ov, lane);
         }
       }
@@ -618,7 +620,8 @@ __device__ __forceinline__ void multi_tile(const MultiArgs &a, const float *__re
 }
 
 template <int K, int FB>
-__global__ void __launch_bounds__(kCtaWarps *kWarp) k_conv2d_multi(const MultiArgs a) {
+// (the explicit 2 CTAs/SM keeps ptxas from capping the registers at 96 and spilling: tests/test_sass.py)
+__global__ void __launch_bounds__(kCtaWarps *kWarp, 2) k_conv2d_multi(const MultiArgs a) {
   constexpr int KP = KCfg<K>::KP;
   extern __shared__ __align__(16) float smem[];
   // CTA = 4 warps on the same (n, F-block): stage that block's filters, layout [C][K][FB][KP]

@@ -214,8 +214,10 @@ __device__ __forceinline__ void multi_tile2(const Multi2Args &a, const MultiFilt
 
 // Tiles are ordered ((group * n_fb + fblk) * n_bands + band) * n_cb + cb; the host pads n_bands so that
 // the CTA's warps share (group, fblk): the CTA stages that F-block's C*K*FB*KP floats once.
-template <int K, int FB, int U, int SEG, int GUARDS, int PF>
-__global__ void __launch_bounds__(kCtaWarps *kWarp, 3) k_conv2d_multi2(const Multi2Args a) {
+// MINB: resident CTAs per SM the register allocation is capped for (3: <= 168 registers). K <= 3 with
+// FB = 8 filters per warp needs more than 168 without spilling: MINB = 2 there (0 LDL/STL, tests/test_sass.py).
+template <int K, int FB, int U, int SEG, int GUARDS, int PF, int MINB = 3>
+__global__ void __launch_bounds__(kCtaWarps *kWarp, MINB) k_conv2d_multi2(const Multi2Args a) {
   constexpr int KP = KCfg<K>::KP;
   extern __shared__ __align__(16) float smem[];
   const long long tile0 = static_cast<long long>(blockIdx.x) * kCtaWarps;

@@ -126,21 +126,45 @@ __device__ __forceinline__ void wide_window(const WideRow &b, float (&w)[WideCfg
   }
 }
 
-// a3: one input row into the ring: acc[q] = acc[q+1] + w . filter[K-1-q] (shift folded into the FMA
-// chains, static indices). GUARD: only slots qmin <= q < qmax (Alg. 2 cases 1 / 3, warp-uniform).
-template <int K, int FSRC, bool GUARD>
-__device__ __forceinline__ void wide_step(float (&acc)[K][kWideV], const float (&w)[WideCfg<K>::WN],
-                                          const FilterSrc<K, FSRC> &fs, int qmin, int qmax) {
+// a4: filter rows of a KH x KW filter (rows padded to KP = ceil(KW/4)*4 floats): the per-K constant slot
+// (uniform registers, square filters) or the CTA's shared-memory copy (broadcast LDS.128).
+template <int KH, int KW, int FSRC>
+struct FilterRows {
+  static constexpr int KP = (KW + 3) / 4 * 4;
+  unsigned sbase;
+  const float *cbase;
+  __device__ __forceinline__ void row(float (&fr)[KP], int i) const {
+    if constexpr (FSRC == FSRC_CONST) {
+      const float4 *p = reinterpret_cast<const float4 *>(cbase + i * KP);
 #pragma unroll
-  for (int q = 0; q < K; ++q) {
+      for (int c = 0; c < KP / 4; ++c) {
+        const float4 v = p[c];
+        fr[4 * c] = v.x; fr[4 * c + 1] = v.y; fr[4 * c + 2] = v.z; fr[4 * c + 3] = v.w;
+      }
+    } else {
+#pragma unroll
+      for (int c = 0; c < KP / 4; ++c)
+        lds4_at(sbase + static_cast<unsigned>((i * KP + 4 * c) * 4), fr[4 * c], fr[4 * c + 1], fr[4 * c + 2],
+                fr[4 * c + 3]);
+    }
+  }
+};
+
+// a3: one input row into the KH-slot ring: acc[q] = acc[q+1] + w . filter[KH-1-q] (shift folded into
+// the FMA chains, static indices). GUARD: only slots qmin <= q < qmax (Alg. 2 cases 1 / 3, warp-uniform).
+template <int KH, int KW, int FSRC, bool GUARD>
+__device__ __forceinline__ void wide_step(float (&acc)[KH][kWideV], const float (&w)[WideCfg<KW>::WN],
+                                          const FilterRows<KH, KW, FSRC> &fs, int qmin, int qmax) {
+#pragma unroll
+  for (int q = 0; q < KH; ++q) {
     if (!GUARD || (q >= qmin && q < qmax)) {
-      float fr[KCfg<K>::KP];
-      fs.row(fr, K - 1 - q);
+      float fr[FilterRows<KH, KW, FSRC>::KP];
+      fs.row(fr, KH - 1 - q);
 #pragma unroll
       for (int v = 0; v < kWideV; ++v) {
-        float s = (q + 1 < K) ? acc[(q + 1 < K) ? q + 1 : 0][v] : 0.f;
+        float s = (q + 1 < KH) ? acc[(q + 1 < KH) ? q + 1 : 0][v] : 0.f;
 #pragma unroll
-        for (int j = 0; j < K; ++j) s = fmaf(w[v + j], fr[j], s);
+        for (int j = 0; j < KW; ++j) s = fmaf(w[v + j], fr[j], s);
         acc[q][v] = s;
       }
     }
@@ -200,21 +224,21 @@ __device__ __forceinline__ void wide_store(float *__restrict__ orow, int x0, int
 // One warp tile: 256 columns x output rows [ob, oe), input rows [ob, oe+K-1) streamed once (Alg. 2's
 // three cases as in single_tile). PF 1 / 2: the next one / two rows in flight in registers; PF >= 3
 // (power of two, EDGE < 2): a PF-stage cp.async ring, PF-1 rows in flight. GUARDS as single_tile.
-template <int K, int FSRC, int PF, int GUARDS, int EDGE, bool HALO>
+template <int KH, int KW, int FSRC, int PF, int GUARDS, int EDGE, bool HALO>
 __device__ __forceinline__ void wide_tile(const SingleArgs &a, const float *__restrict__ inb, float *__restrict__ outb,
-                                          const FilterSrc<K, FSRC> &fs, int x0, int ob, int oe, int lane,
+                                          const FilterRows<KH, KW, FSRC> &fs, int x0, int ob, int oe, int lane,
                                           unsigned ring_base) {
   constexpr bool SAFE = (EDGE != 0);
   constexpr int NST = (PF >= 3 && EDGE != 2) ? PF : 1;
   static_assert(NST == 1 || (NST & (NST - 1)) == 0, "ring depth must be a power of two");
-  const int rend = oe + K - 1;
+  const int rend = oe + KH - 1;
   const int rlast = rend - 1;
-  float acc[K][kWideV];
+  float acc[KH][kWideV];
 #pragma unroll
-  for (int q = 0; q < K; ++q)
+  for (int q = 0; q < KH; ++q)
 #pragma unroll
     for (int v = 0; v < kWideV; ++v) acc[q][v] = 0.f;
-  WideRing<K, (NST > 1 ? NST : 2)> ring;
+  WideRing<KW, (NST > 1 ? NST : 2)> ring;
   ring.base = ring_base;
   ring.lane = lane;
   ring.sl = lane;
@@ -223,8 +247,8 @@ __device__ __forceinline__ void wide_tile(const SingleArgs &a, const float *__re
 #pragma unroll
     for (int st = 0; st < NST - 1; ++st) ring.issue(st, in_row<HALO>(a, inb, min(ob + st, rlast)), x0, a.Wc, EDGE == 1);
   } else {
-    wide_load<K, EDGE>(n1, in_row<HALO>(a, inb, ob), x0, a.Wc, lane);
-    if constexpr (PF == 2) wide_load<K, EDGE>(n2, in_row<HALO>(a, inb, min(ob + 1, rlast)), x0, a.Wc, lane);
+    wide_load<KW, EDGE>(n1, in_row<HALO>(a, inb, ob), x0, a.Wc, lane);
+    if constexpr (PF == 2) wide_load<KW, EDGE>(n2, in_row<HALO>(a, inb, min(ob + 1, rlast)), x0, a.Wc, lane);
   }
   // returns row r and issues the fetch of row r + depth (index clamped). PF == 2: the copy n1 = n2 reads
   // a row fetched one full iteration earlier, so it never waits on the load (PF == 1's cur = n1 copy
@@ -239,10 +263,10 @@ __device__ __forceinline__ void wide_tile(const SingleArgs &a, const float *__re
     } else if constexpr (PF == 2) {
       cur = n1;
       n1 = n2;
-      wide_load<K, EDGE>(n2, in_row<HALO>(a, inb, min(r + 2, rlast)), x0, a.Wc, lane);
+      wide_load<KW, EDGE>(n2, in_row<HALO>(a, inb, min(r + 2, rlast)), x0, a.Wc, lane);
     } else {
       cur = n1;
-      wide_load<K, EDGE>(n1, in_row<HALO>(a, inb, min(r + 1, rlast)), x0, a.Wc, lane);
+      wide_load<KW, EDGE>(n1, in_row<HALO>(a, inb, min(r + 1, rlast)), x0, a.Wc, lane);
     }
     return cur;
   };
@@ -251,50 +275,53 @@ __device__ __forceinline__ void wide_tile(const SingleArgs &a, const float *__re
   if constexpr (GUARDS == 0) {
     for (; r < rend; ++r) {
       const WideRow cur = next_row(r);
-      float w[WideCfg<K>::WN];
-      wide_window<K>(cur, w, lane);
-      wide_step<K, FSRC, false>(acc, w, fs, 0, K);
-      if (r >= ob + K - 1) wide_store<SAFE>(out_at(r - K + 1), x0, a.Wo, acc[0], lane);
+      float w[WideCfg<KW>::WN];
+      wide_window<KW>(cur, w, lane);
+      wide_step<KH, KW, FSRC, false>(acc, w, fs, 0, KH);
+      if (r >= ob + KH - 1) wide_store<SAFE>(out_at(r - KH + 1), x0, a.Wo, acc[0], lane);
     }
     return;
   }
-  for (; r < min(ob + K - 1, oe); ++r) {  // case 1: slots of outputs >= ob only
+  for (; r < min(ob + KH - 1, oe); ++r) {  // case 1: slots of outputs >= ob only
     const WideRow cur = next_row(r);
-    float w[WideCfg<K>::WN];
-    wide_window<K>(cur, w, lane);
-    wide_step<K, FSRC, true>(acc, w, fs, K - 1 - (r - ob), K);
+    float w[WideCfg<KW>::WN];
+    wide_window<KW>(cur, w, lane);
+    wide_step<KH, KW, FSRC, true>(acc, w, fs, KH - 1 - (r - ob), KH);
   }
   const int steady_end = (GUARDS == 2) ? oe : rend;
   for (; r < steady_end; ++r) {  // case 2 (+3 when GUARDS == 1)
     const WideRow cur = next_row(r);
-    float w[WideCfg<K>::WN];
-    wide_window<K>(cur, w, lane);
-    wide_step<K, FSRC, false>(acc, w, fs, 0, K);
-    if (GUARDS == 2 || r >= ob + K - 1) wide_store<SAFE>(out_at(r - K + 1), x0, a.Wo, acc[0], lane);
+    float w[WideCfg<KW>::WN];
+    wide_window<KW>(cur, w, lane);
+    wide_step<KH, KW, FSRC, false>(acc, w, fs, 0, KH);
+    if (GUARDS == 2 || r >= ob + KH - 1) wide_store<SAFE>(out_at(r - KH + 1), x0, a.Wo, acc[0], lane);
   }
   for (; r < rend; ++r) {  // case 3 (GUARDS == 2): slots of outputs < oe only
     const WideRow cur = next_row(r);
-    float w[WideCfg<K>::WN];
-    wide_window<K>(cur, w, lane);
-    wide_step<K, FSRC, true>(acc, w, fs, max(0, K - 1 - (r - ob)), oe + K - 1 - r);
-    if (r >= ob + K - 1) wide_store<SAFE>(out_at(r - K + 1), x0, a.Wo, acc[0], lane);
+    float w[WideCfg<KW>::WN];
+    wide_window<KW>(cur, w, lane);
+    wide_step<KH, KW, FSRC, true>(acc, w, fs, max(0, KH - 1 - (r - ob)), oe + KH - 1 - r);
+    if (r >= ob + KH - 1) wide_store<SAFE>(out_at(r - KH + 1), x0, a.Wo, acc[0], lane);
   }
 }
 
 // One warp per CTA (warp-uniform control flow: the constant-slot filter stays in uniform registers).
-// SingleArgs.n_cb counts 256-column blocks.
-template <int K, int FSRC, int PF, int GUARDS, bool HALO>
-__global__ void __launch_bounds__(kWarp) k_conv2d_wide(const SingleArgs a) {
-  constexpr int KP = KCfg<K>::KP;
-  __shared__ __align__(16) float sf[(FSRC == FSRC_SMEM) ? K * KP : 4];
+// SingleArgs.n_cb counts 256-column blocks. KH x KW filter (square: KH = KW = K; rectangular filters,
+// conv2d_single_rect, take the shared-memory filter).
+template <int KH, int KW, int FSRC, int PF, int GUARDS, bool HALO>
+// Rectangular instantiations state 8 resident CTAs (a 255-register cap): without it ptxas caps some
+// (KH, KW) at 168 registers and spills (tests/test_sass.py); square ones keep ptxas' own choice.
+__global__ void __launch_bounds__(kWarp, (KH != KW) ? 8 : 1) k_conv2d_wide(const SingleArgs a) {
+  using FR = FilterRows<KH, KW, FSRC>;
+  __shared__ __align__(16) float sf[(FSRC == FSRC_SMEM) ? KH * FR::KP : 4];
   extern __shared__ __align__(16) float wide_ring_smem[];
-  FilterSrc<K, FSRC> fs;
+  FR fs;
   if constexpr (FSRC == FSRC_CONST) {
     fs.cbase = c_filt;
   } else {
-    for (int t = threadIdx.x; t < K * KP; t += blockDim.x) {
-      const int i = t / KP, j = t % KP;
-      sf[t] = (j < K) ? a.filt[i * K + j] : 0.f;
+    for (int t = threadIdx.x; t < KH * FR::KP; t += blockDim.x) {
+      const int i = t / FR::KP, j = t % FR::KP;
+      sf[t] = (j < KW) ? a.filt[i * KW + j] : 0.f;
     }
     __syncwarp();
     fs.sbase = static_cast<unsigned>(__cvta_generic_to_shared(sf));
@@ -313,11 +340,11 @@ __global__ void __launch_bounds__(kWarp) k_conv2d_wide(const SingleArgs a) {
   const int oe = band_start(band + 1, a.n_bands, a.Ho);
   const bool inside = x0 + kWideSpan + 16 <= a.W;  // span + both halo quads in range (warp-uniform)
   if (a.aligned && inside)
-    wide_tile<K, FSRC, PF, GUARDS, 0, HALO>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
+    wide_tile<KH, KW, FSRC, PF, GUARDS, 0, HALO>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
   else if (a.aligned)
-    wide_tile<K, FSRC, PF, GUARDS, 1, HALO>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
+    wide_tile<KH, KW, FSRC, PF, GUARDS, 1, HALO>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
   else
-    wide_tile<K, FSRC, PF, GUARDS, 2, HALO>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
+    wide_tile<KH, KW, FSRC, PF, GUARDS, 2, HALO>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
 }
 
 }  // namespace c2d

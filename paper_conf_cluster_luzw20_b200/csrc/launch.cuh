@@ -207,7 +207,7 @@ int launch_single_v(const SingleGeom &g, const float *filt, float *out, cudaStre
 template <int K, int FSRC, int PF, int GUARDS, bool HALO = false>
 int launch_wide_v(const SingleGeom &g, const float *filt, float *out, cudaStream_t stream, int band_h,
                   const DevInfo &dev, int min_band) {
-  auto kernel = k_conv2d_wide<K, FSRC, PF, GUARDS, HALO>;
+  auto kernel = k_conv2d_wide<K, K, FSRC, PF, GUARDS, HALO>;
   static OccCache occ_cache;
   const size_t ring = (PF >= 3) ? WideRing<K, (PF >= 3 ? PF : 2)>::kBytes : 0;
   SingleArgs a;
@@ -224,6 +224,31 @@ int launch_wide_v(const SingleGeom &g, const float *filt, float *out, cudaStream
   };
   if constexpr (FSRC == FSRC_CONST) return with_const_filter(filt, K, KCfg<K>::KP, stream, dev, go);
   return go();
+}
+
+// Rectangular KH x KW filters (conv2d_single_rect): the wide-lane kernel with a KH-slot
+// ring and a KW-wide window, filter staged per CTA in shared memory, one row in flight in registers.
+template <int KH, int KW>
+int launch_rect_v(const float *in, int H, int W, const float *filt, float *out, cudaStream_t stream,
+                  const DevInfo &dev) {
+  auto kernel = k_conv2d_wide<KH, KW, FSRC_SMEM, 1, 0, false>;
+  static OccCache occ_cache;
+  SingleArgs a;
+  const SingleGeom g{in, in, 1, H, W, H, W, W - KW + 1};
+  fill_args(a, g, KH, 2, out);  // Ho from KH
+  a.Wo = W - KW + 1;
+  a.img_out = static_cast<long long>(a.Ho) * a.Po;
+  a.n_cb = ceil_div(a.Wo, kWideSpan);
+  a.filt = filt;
+  const long long resident = static_cast<long long>(cta_occupancy(kernel, 0, occ_cache, kWarp)) * dev.num_sms;
+  const bool tiny = static_cast<long long>(H) * W <= 512LL * 512;
+  const int min_band = tiny ? 1 : (KH - 1 > 4 ? KH - 1 : 4);
+  a.n_bands = band_count(a.Ho, KH, a.n_cb, 1, resident, 0, min_band);
+  const long long tiles = static_cast<long long>(a.n_cb) * a.n_bands;
+  if (tiles > 0x7fffffffLL) return CONV2D_ESHAPE;
+  a.n_tiles = static_cast<int>(tiles);
+  kernel<<<a.n_tiles, kWarp, 0, stream>>>(a);
+  return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
 }
 
 // Filter-row split (conv2d_split.cuh): same tile geometry as launch_single_v, but a tile takes G
@@ -483,12 +508,12 @@ int launch_multi_fb(const float *in, int N, int C, int H, int W, const float *fi
   return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
 }
 
-template <int K, int FB, int U, int SEG, int GUARDS, int PF>
+template <int K, int FB, int U, int SEG, int GUARDS, int PF, int MINB = (K <= 3 && FB * U >= 8) ? 2 : 3>
 int launch_multi2_v(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
                     cudaStream_t stream, int band_h, const DevInfo &dev) {
   constexpr int KP = KCfg<K>::KP;
   constexpr int SEGS = kWarp / SEG;
-  auto kernel = k_conv2d_multi2<K, FB, U, SEG, GUARDS, PF>;
+  auto kernel = k_conv2d_multi2<K, FB, U, SEG, GUARDS, PF, MINB>;
   static OccCache occ_cache;
   static SmemOptIn smem_flag;
   const size_t ring = (PF >= 3) ? kCtaWarps * RowRing<K, U, SEG, PF>::kBytes : 0;
@@ -670,6 +695,10 @@ int launch_multi(const float *in, int N, int C, int H, int W, const float *filt,
   if (mv == 3) return C2D_LM(FBH, 32);
   if (mv == 4) return C2D_LM(FBH, 16);
   if (mv == 7) return (K > 3) ? C2D_LM(FBH, 8) : C2D_LM(FB, 8);
+  // the pre-r02 register cap (3 CTAs per SM) for the FB = 8 kernels (spills at K <= 3)
+  if (mv == 70) return launch_multi2_v<K, FB, 1, 16, GUARDS, PF, 3>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
+  if (mv == 71) return launch_multi2_v<K, FB, 1, 8, GUARDS, PF, 3>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
+  if (mv == 72) return launch_multi2_v<K, FB, 1, 32, GUARDS, PF, 3>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
 #undef C2D_LM2
   {
     // wide-lane kernel (conv2d_mwide.cuh), variants 60-69: SEG x {PF 1, 2}
@@ -725,6 +754,19 @@ template <int K>
 int multi_entry(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
                 cudaStream_t stream, int band_h, const DevInfo &dev) {
   return launch_multi<K>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
+}
+
+template <int KH>
+int rect_entry(const float *in, int H, int W, const float *filt, int KW, float *out, cudaStream_t stream,
+               const DevInfo &dev) {
+  switch (KW) {
+#define C2D_RECT(KK) \
+  case KK: return launch_rect_v<KH, KK>(in, H, W, filt, out, stream, dev);
+    C2D_RECT(1) C2D_RECT(2) C2D_RECT(3) C2D_RECT(4) C2D_RECT(5) C2D_RECT(6) C2D_RECT(7) C2D_RECT(8)
+    C2D_RECT(9) C2D_RECT(10) C2D_RECT(11) C2D_RECT(12) C2D_RECT(13) C2D_RECT(14) C2D_RECT(15)
+#undef C2D_RECT
+    default: return CONV2D_EK;
+  }
 }
 
 }  // namespace c2d

@@ -130,6 +130,12 @@ def test_batch_argument_errors_need_no_gpu(lib):
     # the second image's input (bytes 256..512) overlaps the output
     assert c.conv2d_single_batch(a, 2, 8, 8, b, 3, a + 300) == c.CONV2D_EOVERLAP
     assert c.conv2d_multi_tc(a, 2, 2, 8, 8, b, 1, 3, a + 100) == c.CONV2D_EOVERLAP
+    # conv2d_single_rect (N4): FH x FW in [1, 15]
+    assert c.conv2d_single_rect(None, 8, 8, b, 3, 5, o) == c.CONV2D_ENULL
+    assert c.conv2d_single_rect(a, 8, 8, b, 3, 16, o) == c.CONV2D_EK
+    assert c.conv2d_single_rect(a, 8, 8, b, 0, 5, o) == c.CONV2D_ESHAPE
+    assert c.conv2d_single_rect(a, 8, 4, b, 3, 5, o) == c.CONV2D_ESHAPE
+    assert c.conv2d_single_rect(a, 8, 8, b, 3, 5, a + 16) == c.CONV2D_EOVERLAP
 
 
 def test_product_library_has_no_tuning_switches(lib):
