@@ -214,9 +214,12 @@ __device__ __forceinline__ void multi_tile2(const Multi2Args &a, const MultiFilt
 
 // Tiles are ordered ((group * n_fb + fblk) * n_bands + band) * n_cb + cb; the host pads n_bands so that
 // the CTA's warps share (group, fblk): the CTA stages that F-block's C*K*FB*KP floats once.
-// MINB: resident CTAs per SM the register allocation is capped for (3: <= 168 registers). K <= 3 with
-// FB = 8 filters per warp needs more than 168 without spilling: MINB = 2 there (0 LDL/STL, tests/test_sass.py).
-template <int K, int FB, int U, int SEG, int GUARDS, int PF, int MINB = 3>
+// MINB: resident CTAs per SM the register allocation is capped for (3: <= 168 registers; whole-warp
+// rows with FB = 8 at K <= 3 need more: MINB = 2 there). ALIGNED: the launch's input is 16-byte aligned
+// with W % 4 == 0 (interior + ragged-edge tiles); the misaligned case (guarded scalar loads) is its own
+// instantiation, so its register demand never caps -- or spills in -- the hot kernel (0 LDL/STL,
+// tests/test_sass.py).
+template <int K, int FB, int U, int SEG, int GUARDS, int PF, int MINB = 3, bool ALIGNED = true>
 __global__ void __launch_bounds__(kCtaWarps *kWarp, MINB) k_conv2d_multi2(const Multi2Args a) {
   constexpr int KP = KCfg<K>::KP;
   extern __shared__ __align__(16) float smem[];
@@ -254,12 +257,14 @@ __global__ void __launch_bounds__(kCtaWarps *kWarp, MINB) k_conv2d_multi2(const 
   const bool seg_active = n_raw < a.N;
   const int n = seg_active ? n_raw : a.N - 1;  // idle segments recompute the last image, never store
   const bool inside = x0 + 4 * SEG * U + 4 * KCfg<K>::NE <= a.W;  // uniform per warp
-  if (a.aligned && inside)
-    multi_tile2<K, FB, U, SEG, GUARDS, PF, 0>(a, mf, n, seg_active, f0, x0, ob, oe, lane, ring_base);
-  else if (a.aligned)
-    multi_tile2<K, FB, U, SEG, GUARDS, PF, 1>(a, mf, n, seg_active, f0, x0, ob, oe, lane, ring_base);
-  else
+  if constexpr (ALIGNED) {
+    if (inside)
+      multi_tile2<K, FB, U, SEG, GUARDS, PF, 0>(a, mf, n, seg_active, f0, x0, ob, oe, lane, ring_base);
+    else
+      multi_tile2<K, FB, U, SEG, GUARDS, PF, 1>(a, mf, n, seg_active, f0, x0, ob, oe, lane, ring_base);
+  } else {
     multi_tile2<K, FB, U, SEG, GUARDS, PF, 2>(a, mf, n, seg_active, f0, x0, ob, oe, lane, ring_base);
+  }
 }
 
 }  // namespace c2d

@@ -15,7 +15,6 @@
 #include "conv2d_multi.cuh"
 #include "conv2d_split.cuh"
 #include "conv2d_wide.cuh"
-#include "conv2d_mwide.cuh"
 
 namespace {
 
@@ -177,11 +176,11 @@ void fill_args(ArgsT &a, const SingleGeom &g, int K, int U, float *out) {
   a.aligned = (aligned16(g.in) && aligned16(g.in2) && (g.P % 4 == 0)) ? 1 : 0;
 }
 
-template <int K, int U, int FSRC, int PF = 1, int GUARDS = 0, bool HALO = false>
+template <int K, int U, int FSRC, int PF = 1, int GUARDS = 0, bool HALO = false, int L2D = 0>
 int launch_single_v(const SingleGeom &g, const float *filt, float *out, cudaStream_t stream, int band_h,
                     const DevInfo &dev, int min_band) {
   constexpr int CTAW = (FSRC == FSRC_CONST) ? 1 : kCtaWarps;
-  auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS, HALO>;
+  auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS, HALO, L2D>;
   static OccCache occ_cache;
   const size_t ring = (PF >= 3) ? CTAW * RowRing<K, U, kWarp, (PF >= 3 ? PF : 2)>::kBytes : 0;
   SingleArgs a;
@@ -204,10 +203,10 @@ int launch_single_v(const SingleGeom &g, const float *filt, float *out, cudaStre
 
 // Wide-lane kernel (conv2d_wide.cuh): 8 contiguous columns per lane, 256-column warp tiles, one warp
 // per CTA.
-template <int K, int FSRC, int PF, int GUARDS, bool HALO = false>
+template <int K, int FSRC, int PF, int GUARDS, bool HALO = false, int L2D = 0>
 int launch_wide_v(const SingleGeom &g, const float *filt, float *out, cudaStream_t stream, int band_h,
                   const DevInfo &dev, int min_band) {
-  auto kernel = k_conv2d_wide<K, K, FSRC, PF, GUARDS, HALO>;
+  auto kernel = k_conv2d_wide<K, K, FSRC, PF, GUARDS, HALO, L2D>;
   static OccCache occ_cache;
   const size_t ring = (PF >= 3) ? WideRing<K, (PF >= 3 ? PF : 2)>::kBytes : 0;
   SingleArgs a;
@@ -434,6 +433,15 @@ int launch_single(const SingleGeom &g, const float *filt, float *out, cudaStream
     case 27: if (constant_ok) return C2D_LW(FSRC_CONST, 2, 0); break;
     case 28: if (constant_ok) return C2D_LW(FSRC_CONST, 2, 2); break;
     case 29: return C2D_LW(FSRC_SMEM, 2, 0);
+    // L2 bulk prefetch of the row L2D ahead (prefetch_l2), on the default kernels' shapes
+    case 30: if (constant_ok) return launch_wide_v<K, FSRC_CONST, 1, 2, false, 4>(g, filt, out, stream, band_h, dev, min_band); break;
+    case 31: if (constant_ok) return launch_wide_v<K, FSRC_CONST, 1, 2, false, 8>(g, filt, out, stream, band_h, dev, min_band); break;
+    case 32: return launch_wide_v<K, FSRC_SMEM, 1, 0, false, 4>(g, filt, out, stream, band_h, dev, min_band);
+    case 33: if (constant_ok) return launch_single_v<K, 1, FSRC_CONST, 1, 1, false, 4>(g, filt, out, stream, band_h, dev, min_band); break;
+    case 34: if (constant_ok) return launch_single_v<K, 1, FSRC_CONST, 1, 1, false, 8>(g, filt, out, stream, band_h, dev, min_band); break;
+    case 35: if (constant_ok) return launch_single_v<K, 1, FSRC_CONST, 4, 1, false, 4>(g, filt, out, stream, band_h, dev, min_band); break;
+    case 36: if (constant_ok) return launch_single_v<K, 2, FSRC_CONST, 4, 0, false, 4>(g, filt, out, stream, band_h, dev, min_band); break;
+    case 37: if (constant_ok) return launch_single_v<K, 1, FSRC_CONST, 4, 2, false, 4>(g, filt, out, stream, band_h, dev, min_band); break;
     default: break;
   }
 #undef C2D_LW
@@ -508,79 +516,6 @@ int launch_multi_fb(const float *in, int N, int C, int H, int W, const float *fi
   return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
 }
 
-template <int K, int FB, int U, int SEG, int GUARDS, int PF, int MINB = (K <= 3 && FB * U >= 8) ? 2 : 3>
-int launch_multi2_v(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
-                    cudaStream_t stream, int band_h, const DevInfo &dev) {
-  constexpr int KP = KCfg<K>::KP;
-  constexpr int SEGS = kWarp / SEG;
-  auto kernel = k_conv2d_multi2<K, FB, U, SEG, GUARDS, PF, MINB>;
-  static OccCache occ_cache;
-  static SmemOptIn smem_flag;
-  const size_t ring = (PF >= 3) ? kCtaWarps * RowRing<K, U, SEG, PF>::kBytes : 0;
-  const size_t smem = static_cast<size_t>(C) * K * FB * KP * sizeof(float) + ring;
-  if (int e = ensure_smem(kernel, smem, dev, smem_flag)) return e;
-  Multi2Args a;
-  a.in = in;
-  a.filt = filt;
-  a.out = out;
-  a.N = N;
-  a.C = C;
-  a.H = H;
-  a.W = W;
-  a.F = F;
-  a.Ho = H - K + 1;
-  a.Wo = W - K + 1;
-  a.n_cb = ceil_div(a.Wo, 4 * SEG * U);
-  a.n_fb = ceil_div(F, FB);
-  a.n_groups = ceil_div(N, SEGS);
-  a.aligned = (aligned16(in) && (W % 4 == 0)) ? 1 : 0;
-  if (band_h <= 0 && K >= 5) {
-    // one full wave of resident warps (tools/multi_band_sweep.py: for K >= 5 the K-1 prologue rows
-    // of extra bands cost more than the wave quantisation they remove -- Table I CONV3/CONV5, configs[3])
-    const long long resident_warps =
-        static_cast<long long>(cta_occupancy(kernel, smem, occ_cache, kCtaWarps * kWarp)) * kCtaWarps * dev.num_sms;
-    const long long groups = static_cast<long long>(a.n_groups) * a.n_fb * a.n_cb;
-    long long bands = resident_warps / groups;
-    if (bands < 1) bands = 1;
-    band_h = ceil_div(a.Ho, bands);
-  } else if (band_h <= 0) {
-    // K <= 4: band count by a wave-quantisation cost model: a tile of h output rows streams h + K - 1
-    // input rows, and the grid runs in ceil(CTAs / resident CTAs) waves, so pick the band count b
-    // that minimises waves(b) * (ceil(Ho / b) + K - 1). (One band per tile whenever the (image,
-    // F-block, column-block) groups alone exceed a wave left e.g. Table I CONV11 at 1.15 waves -- 2
-    // waves, the second 15% full: 946 -> 570 us; CONV8/9 2x.)
-    const long long resident_ctas = static_cast<long long>(cta_occupancy(kernel, smem, occ_cache, kCtaWarps * kWarp)) * dev.num_sms;
-    const long long groups = static_cast<long long>(a.n_groups) * a.n_fb;
-    long long best_b = 1;
-    double best = 1e300;
-    const int bmax = a.Ho < 512 ? a.Ho : 512;
-    for (int b = 1; b <= bmax; ++b) {
-      const int h = ceil_div(a.Ho, b);
-      const int nb = ceil_div(a.Ho, h);  // bands actually used with height h
-      long long nbp = nb;
-      while ((static_cast<long long>(a.n_cb) * nbp) % kCtaWarps) ++nbp;
-      const long long ctas = groups * a.n_cb * nbp / kCtaWarps;
-      const long long waves = (ctas + resident_ctas - 1) / resident_ctas;
-      const double cost = static_cast<double>(waves) * (h + K - 1) * (1.0 + 1e-3 * (nbp - nb));
-      if (cost < best - 1e-9) {
-        best = cost;
-        best_b = nb;
-      }
-    }
-    band_h = ceil_div(a.Ho, best_b);
-  }
-  if (band_h > a.Ho) band_h = a.Ho;
-  a.band_h = band_h;
-  int n_bands = ceil_div(a.Ho, band_h);
-  while ((static_cast<long long>(a.n_cb) * n_bands) % kCtaWarps) ++n_bands;
-  a.n_bands = n_bands;
-  a.n_tiles = static_cast<long long>(a.n_groups) * a.n_fb * n_bands * a.n_cb;
-  const long long blocks = (a.n_tiles + kCtaWarps - 1) / kCtaWarps;
-  if (blocks > 0x7fffffffLL) return CONV2D_ESHAPE;
-  kernel<<<static_cast<unsigned>(blocks), kCtaWarps * kWarp, smem, stream>>>(a);
-  return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
-}
-
 // Multi-channel band choice shared by the multi kernels: K >= 5 one full wave of resident warps (the
 // K-1 prologue rows of extra bands cost more than the wave quantisation they remove --
 // tools/multi_band_sweep.py: Table I CONV3/CONV5, configs[3]); K <= 4 the wave-quantisation cost model
@@ -619,17 +554,16 @@ int multi_bands(int Ho, int n_cb, long long groups, long long resident_ctas, int
   return n_bands;
 }
 
-// Wide-lane multi-channel kernel (conv2d_mwide.cuh): FB filters per warp, SEG-lane segments of 8*SEG
-// columns, PF (row, channel) entries in flight in registers.
-template <int K, int FB, int SEG, int GUARDS, int PF, int MINB>
-int launch_mwide_v(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
-                   cudaStream_t stream, int band_h, const DevInfo &dev) {
+template <int K, int FB, int U, int SEG, int GUARDS, int PF, int MINB, bool ALIGNED>
+int launch_multi2_k(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
+                    cudaStream_t stream, int band_h, const DevInfo &dev) {
   constexpr int KP = KCfg<K>::KP;
   constexpr int SEGS = kWarp / SEG;
-  auto kernel = k_conv2d_mwide<K, FB, SEG, GUARDS, PF, MINB>;
+  auto kernel = k_conv2d_multi2<K, FB, U, SEG, GUARDS, PF, MINB, ALIGNED>;
   static OccCache occ_cache;
   static SmemOptIn smem_flag;
-  const size_t smem = static_cast<size_t>(C) * K * FB * KP * sizeof(float);
+  const size_t ring = (PF >= 3) ? kCtaWarps * RowRing<K, U, SEG, PF>::kBytes : 0;
+  const size_t smem = static_cast<size_t>(C) * K * FB * KP * sizeof(float) + ring;
   if (int e = ensure_smem(kernel, smem, dev, smem_flag)) return e;
   Multi2Args a;
   a.in = in;
@@ -642,20 +576,31 @@ int launch_mwide_v(const float *in, int N, int C, int H, int W, const float *fil
   a.F = F;
   a.Ho = H - K + 1;
   a.Wo = W - K + 1;
-  a.n_cb = ceil_div(a.Wo, kWideV * SEG);
+  a.n_cb = ceil_div(a.Wo, 4 * SEG * U);
   a.n_fb = ceil_div(F, FB);
   a.n_groups = ceil_div(N, SEGS);
   a.aligned = (aligned16(in) && (W % 4 == 0)) ? 1 : 0;
   const long long resident_ctas =
       static_cast<long long>(cta_occupancy(kernel, smem, occ_cache, kCtaWarps * kWarp)) * dev.num_sms;
-  a.n_bands = multi_bands<K>(a.Ho, a.n_cb, static_cast<long long>(a.n_groups) * a.n_fb, resident_ctas, band_h);
+  const int n_bands = multi_bands<K>(a.Ho, a.n_cb, static_cast<long long>(a.n_groups) * a.n_fb, resident_ctas, band_h);
   a.band_h = band_h;
-  a.n_tiles = static_cast<long long>(a.n_groups) * a.n_fb * a.n_bands * a.n_cb;
+  a.n_bands = n_bands;
+  a.n_tiles = static_cast<long long>(a.n_groups) * a.n_fb * n_bands * a.n_cb;
   const long long blocks = (a.n_tiles + kCtaWarps - 1) / kCtaWarps;
   if (blocks > 0x7fffffffLL) return CONV2D_ESHAPE;
   kernel<<<static_cast<unsigned>(blocks), kCtaWarps * kWarp, smem, stream>>>(a);
   return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
 }
+
+template <int K, int FB, int U, int SEG, int GUARDS, int PF, int MINB = (SEG == kWarp && K <= 3 && FB * U >= 8) ? 2 : 3>
+int launch_multi2_v(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
+                    cudaStream_t stream, int band_h, const DevInfo &dev) {
+  const bool aligned = aligned16(in) && (W % 4 == 0);
+  if (!aligned)  // the misaligned-input instantiation (guarded scalar loads), its own register budget
+    return launch_multi2_k<K, FB, U, SEG, GUARDS, PF, 2, false>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
+  return launch_multi2_k<K, FB, U, SEG, GUARDS, PF, MINB, true>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
+}
+
 
 // fraction of a segment-row's lanes doing valid columns
 inline double lane_use(int Wo, int span) { return double(Wo) / (double(ceil_div(Wo, span)) * span); }
@@ -700,24 +645,6 @@ int launch_multi(const float *in, int N, int C, int H, int W, const float *filt,
   if (mv == 71) return launch_multi2_v<K, FB, 1, 8, GUARDS, PF, 3>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
   if (mv == 72) return launch_multi2_v<K, FB, 1, 32, GUARDS, PF, 3>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
 #undef C2D_LM2
-  {
-    // wide-lane kernel (conv2d_mwide.cuh), variants 60-69: SEG x {PF 1, 2}
-    constexpr int FBW = (K <= 3) ? 4 : (K <= 8 ? 2 : 1);
-#define C2D_LMW(SEGG, PFF) \
-  launch_mwide_v<K, FBW, SEGG, GUARDS, PFF, 2>(in, N, C, H, W, filt, F, out, stream, band_h, dev)
-    switch (mv) {
-      case 60: return C2D_LMW(32, 1);
-      case 61: return C2D_LMW(32, 2);
-      case 62: return C2D_LMW(16, 1);
-      case 63: return C2D_LMW(16, 2);
-      case 64: return C2D_LMW(8, 1);
-      case 65: return C2D_LMW(8, 2);
-      case 66: return C2D_LMW(4, 1);
-      case 67: return C2D_LMW(4, 2);
-      default: break;
-    }
-#undef C2D_LMW
-  }
 #endif
   // Tuned on B200 (tools/multi_variants.py): 16-lane segments (two images per warp) unless they waste
   // clearly more lanes than whole-warp rows -- more column blocks take the vector fast path and the

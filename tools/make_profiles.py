@@ -23,12 +23,18 @@ import ncu_raw_summary  # noqa: E402
 
 # ncu capture name -> bench point name (tools/gpu_round.sh profiles these configurations)
 CAPTURES = {
+    "prof_k15_b8_s8192": "conv2d_single 8192^2 K=15 x8 images",
+    "prof_k3_b8_s8192": "conv2d_single 8192^2 K=3 x8 images",
+    "prof_k7_b8_s8192": "conv2d_single 8192^2 K=7 x8 images",
     "prof_k15_v0_s8192": "conv2d_single 8192^2 K=15",
     "prof_k3_v0_s8192": "conv2d_single 8192^2 K=3",
+    "prof_k7_v0_s8192": "conv2d_single 8192^2 K=7",
+    "prof_k15_s4096": "conv2d_single 4096^2 K=15",
+    "prof_k5_s2048": "conv2d_single 2048^2 K=5",
     "prof_direct_k3_s8192": "conv2d_single_direct 8192^2 K=3 (Fig. 1a baseline)",
     "prof_tc_config2": "conv2d_multi_tc N32 C64 F64 56^2 K3",
     "prof_tc_config3": "conv2d_multi_tc N128 C3 F64 224^2 K7",
-    "prof_k7_v0_s8192": "conv2d_single 8192^2 K=7",
+    "prof_multi_config3": "conv2d_multi N128 C3 F64 224^2 K7",
     "prof_split_k15_s1024": "conv2d_single 1024^2 K=15 (filter-row split, cluster of 2 CTAs)",
     "prof_conv11c1": "conv2d_multi Table I CONV11 C1 N128 224^2 F64 K3",
 }

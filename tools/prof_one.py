@@ -29,6 +29,7 @@ def main():
     ap.add_argument("--variant", type=int, default=0)
     ap.add_argument("--mvariant", type=int, default=0)
     ap.add_argument("--tc", action="store_true", help="multi: the tensor-core variant conv2d_multi_tc")
+    ap.add_argument("--batch", type=int, default=1, help="single: images per call (conv2d_single_batch)")
     a = ap.parse_args()
     pkg._capi.debug_set_variant(a.variant)
     pkg._capi.debug_set_multi_variant(a.mvariant)
@@ -36,10 +37,15 @@ def main():
     if a.kind == "single":
         S = [int(v) for v in a.shape.split(",")]
         H, W = (S[0], S[0]) if len(S) == 1 else S
-        x = synth.fill_torch(1, 1, (H, W), "img", device=dev)
+        x = synth.fill_torch(1, 1, (a.batch, H, W), "img", device=dev)
         f = torch.from_numpy(synth.make_filter(1, a.K, "rand")[0, 0]).to(dev)
-        fn = (lambda: pkg.conv2d_single_direct(x, f)) if a.direct else (lambda: pkg.conv2d_single(x, f, band_h=a.band))
-        px = (H - a.K + 1) * (W - a.K + 1)
+        if a.direct:
+            fn = lambda: pkg.conv2d_single_direct(x[0], f)  # noqa: E731
+        elif a.batch > 1:
+            fn = lambda: pkg.conv2d_single_batch(x, f)  # noqa: E731
+        else:
+            fn = lambda: pkg.conv2d_single(x[0], f, band_h=a.band)  # noqa: E731
+        px = (H - a.K + 1) * (W - a.K + 1) * a.batch
         work = px
     else:
         N, C, H, W, F = [int(v) for v in a.shape.split(",")]
