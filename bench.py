@@ -544,7 +544,7 @@ def run_ours(args):
     roof["peak_source"] = (peaks["source"] if dkind == "hbm" or roof["bound"] == "tensor" else
                            f"fp32 FMA: 148 SM x 128 lanes x 2 x {sm_mhz_peak:.0f} MHz (sm_max_mhz, "
                            f"{peaks['source']})")
-    roof["traffic"] = load_traffic(dp)
+    roof["traffic"] = load_traffic(roof["kernel"])
 
     sweep = []
     for i, p in enumerate(points):
@@ -716,13 +716,14 @@ def _run_e2e(points, unit, args, device):
                      f"conv2d_multi_host (impl={args.multi_impl}; pinned host buffers, 2 streams)")}
 
 
-def load_traffic(p):
-    """dram bytes (read + write) per launch of this kernel config from the committed ncu capture."""
+def load_traffic(kernel_name):
+    """dram bytes (read + write) per launch of this kernel config (bench roofline "kernel" name) from the
+    committed ncu capture (profiles/ncu_traffic.json, tools/make_profiles.py)."""
     path = os.path.join(ROOT, "profiles", "ncu_traffic.json")
     try:
         with open(path) as fh:
             d = json.load(fh)
-        return d.get(f"conv2d_{p.kind} {p.name}")
+        return d.get(kernel_name)
     except Exception:
         return None
 

@@ -118,13 +118,6 @@ __device__ __forceinline__ void load_row_g(RowBuf<K, U> &b, const float *__restr
   }
 }
 
-// L2 bulk prefetch (sm_90+ cp.async.bulk.prefetch.L2): one lane asks the L2 to fetch a 16-byte-aligned
-// range (a tile's row segment) that a later iteration will load -- no registers, no shared memory, one
-// instruction per row per warp; the later LDG then hits L2 instead of waiting for HBM.
-__device__ __forceinline__ void prefetch_l2(const void *g, unsigned bytes) {
-  asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(g), "r"(bytes) : "memory");
-}
-
 // cp.async (LDGSTS) row ring: each lane copies its own quads global -> shared and later reads back
 // only what it wrote itself, so deep prefetch costs no registers, no register copies and no
 // cross-lane synchronisation (cp.async.wait_group per thread is enough).
@@ -400,7 +393,7 @@ __device__ __forceinline__ const float *in_row(const SingleArgs &a, const float 
 // loads, masked scalar stores); 2: misaligned rows (guarded scalar loads, masked stores).
 // PF 1/2: rows r+1 (r+2) in flight in registers; PF >= 3 (power of two, EDGE < 2): a PF-stage cp.async
 // ring in shared memory with PF-1 rows in flight (latency-bound short bands and HBM-bound small K).
-template <int K, int U, int FSRC, int PF, int GUARDS, int EDGE, bool HALO, int L2D = 0>
+template <int K, int U, int FSRC, int PF, int GUARDS, int EDGE, bool HALO>
 __device__ __forceinline__ void single_tile(const SingleArgs &a, const float *__restrict__ inb,
                                             float *__restrict__ outb, const FilterSrc<K, FSRC> &fs, int x0, int ob,
                                             int oe, int lane, unsigned ring_base) {
@@ -430,13 +423,8 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const float *__
     load_row<K, U, SAFE>(n1, in_row<HALO>(a, inb, ob), x0, a.Wc, lane, a.aligned);
     if (RPF == 2) load_row<K, U, SAFE>(n2, in_row<HALO>(a, inb, min(ob + 1, rlast)), x0, a.Wc, lane, a.aligned);
   }
-  // returns row r and issues the fetch of row r+depth (index clamped); L2D > 0 (interior tiles): lane 0
-  // also prefetches row r+L2D's segment into L2
+  // returns row r and issues the fetch of row r+depth (index clamped)
   auto next_row = [&](int r) {
-    if constexpr (L2D > 0 && EDGE == 0 && !HALO) {
-      if (lane == 0 && r + L2D < rend)
-        prefetch_l2(inb + static_cast<size_t>(r + L2D) * a.P + x0, (128 * U + 4 * KCfg<K>::NE) * 4);
-    }
     RowBuf<K, U> cur;
     if constexpr (NST > 1) {
       cp_async_wait<NST - 2>();
@@ -490,7 +478,7 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const float *__
 // CTAW: warps per CTA. With CTAW == 1 every branch depends only on blockIdx and kernel parameters,
 // so the compiler can prove warp-uniform control flow and keep the constant-bank filter in uniform
 // registers (LDCU + FFMA with UR operands) instead of per-lane loads.
-template <int K, int U, int FSRC, int CTAW, int PF = 1, int GUARDS = 0, bool HALO = false, int L2D = 0>
+template <int K, int U, int FSRC, int CTAW, int PF = 1, int GUARDS = 0, bool HALO = false>
 __global__ void __launch_bounds__(CTAW *kWarp) k_conv2d_single(const SingleArgs a) {
   constexpr int KP = KCfg<K>::KP;
   __shared__ __align__(16) float sf[(FSRC == FSRC_SMEM) ? K * KP : 4];
@@ -524,7 +512,7 @@ __global__ void __launch_bounds__(CTAW *kWarp) k_conv2d_single(const SingleArgs 
   // fast tiles: 16B-aligned rows, every column of the tile and its extra halo quad in range
   const bool inside = x0 + 128 * U + 4 * KCfg<K>::NE <= a.W;  // warp-uniform
   if (a.aligned && inside)
-    single_tile<K, U, FSRC, PF, GUARDS, 0, HALO, L2D>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
+    single_tile<K, U, FSRC, PF, GUARDS, 0, HALO>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
   else if (a.aligned)
     single_tile<K, U, FSRC, PF, GUARDS, 1, HALO>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
   else

@@ -224,7 +224,7 @@ __device__ __forceinline__ void wide_store(float *__restrict__ orow, int x0, int
 // One warp tile: 256 columns x output rows [ob, oe), input rows [ob, oe+K-1) streamed once (Alg. 2's
 // three cases as in single_tile). PF 1 / 2: the next one / two rows in flight in registers; PF >= 3
 // (power of two, EDGE < 2): a PF-stage cp.async ring, PF-1 rows in flight. GUARDS as single_tile.
-template <int KH, int KW, int FSRC, int PF, int GUARDS, int EDGE, bool HALO, int L2D = 0>
+template <int KH, int KW, int FSRC, int PF, int GUARDS, int EDGE, bool HALO>
 __device__ __forceinline__ void wide_tile(const SingleArgs &a, const float *__restrict__ inb, float *__restrict__ outb,
                                           const FilterRows<KH, KW, FSRC> &fs, int x0, int ob, int oe, int lane,
                                           unsigned ring_base) {
@@ -254,9 +254,6 @@ __device__ __forceinline__ void wide_tile(const SingleArgs &a, const float *__re
   // a row fetched one full iteration earlier, so it never waits on the load (PF == 1's cur = n1 copy
   // stalls on a load issued late in the previous iteration -- ncu long_scoreboard at that MOV).
   auto next_row = [&](int r) {
-    if constexpr (L2D > 0 && EDGE == 0 && !HALO) {  // lane 0: row r+L2D's segment into L2 (prefetch_l2)
-      if (lane == 0 && r + L2D < rend) prefetch_l2(inb + static_cast<size_t>(r + L2D) * a.P + x0, (kWideSpan + 16) * 4);
-    }
     WideRow cur;
     if constexpr (NST > 1) {
       cp_async_wait<NST - 2>();
@@ -311,7 +308,7 @@ __device__ __forceinline__ void wide_tile(const SingleArgs &a, const float *__re
 // One warp per CTA (warp-uniform control flow: the constant-slot filter stays in uniform registers).
 // SingleArgs.n_cb counts 256-column blocks. KH x KW filter (square: KH = KW = K; rectangular filters,
 // conv2d_single_rect, take the shared-memory filter).
-template <int KH, int KW, int FSRC, int PF, int GUARDS, bool HALO, int L2D = 0>
+template <int KH, int KW, int FSRC, int PF, int GUARDS, bool HALO>
 // Rectangular instantiations state 8 resident CTAs (a 255-register cap): without it ptxas caps some
 // (KH, KW) at 168 registers and spills (tests/test_sass.py); square ones keep ptxas' own choice.
 __global__ void __launch_bounds__(kWarp, (KH != KW) ? 8 : 1) k_conv2d_wide(const SingleArgs a) {
@@ -343,7 +340,7 @@ __global__ void __launch_bounds__(kWarp, (KH != KW) ? 8 : 1) k_conv2d_wide(const
   const int oe = band_start(band + 1, a.n_bands, a.Ho);
   const bool inside = x0 + kWideSpan + 16 <= a.W;  // span + both halo quads in range (warp-uniform)
   if (a.aligned && inside)
-    wide_tile<KH, KW, FSRC, PF, GUARDS, 0, HALO, L2D>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
+    wide_tile<KH, KW, FSRC, PF, GUARDS, 0, HALO>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
   else if (a.aligned)
     wide_tile<KH, KW, FSRC, PF, GUARDS, 1, HALO>(a, inb, outb, fs, x0, ob, oe, lane, ring_base);
   else

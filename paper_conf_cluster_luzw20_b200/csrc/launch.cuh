@@ -176,11 +176,11 @@ void fill_args(ArgsT &a, const SingleGeom &g, int K, int U, float *out) {
   a.aligned = (aligned16(g.in) && aligned16(g.in2) && (g.P % 4 == 0)) ? 1 : 0;
 }
 
-template <int K, int U, int FSRC, int PF = 1, int GUARDS = 0, bool HALO = false, int L2D = 0>
+template <int K, int U, int FSRC, int PF = 1, int GUARDS = 0, bool HALO = false>
 int launch_single_v(const SingleGeom &g, const float *filt, float *out, cudaStream_t stream, int band_h,
                     const DevInfo &dev, int min_band) {
   constexpr int CTAW = (FSRC == FSRC_CONST) ? 1 : kCtaWarps;
-  auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS, HALO, L2D>;
+  auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS, HALO>;
   static OccCache occ_cache;
   const size_t ring = (PF >= 3) ? CTAW * RowRing<K, U, kWarp, (PF >= 3 ? PF : 2)>::kBytes : 0;
   SingleArgs a;
@@ -203,10 +203,10 @@ int launch_single_v(const SingleGeom &g, const float *filt, float *out, cudaStre
 
 // Wide-lane kernel (conv2d_wide.cuh): 8 contiguous columns per lane, 256-column warp tiles, one warp
 // per CTA.
-template <int K, int FSRC, int PF, int GUARDS, bool HALO = false, int L2D = 0>
+template <int K, int FSRC, int PF, int GUARDS, bool HALO = false>
 int launch_wide_v(const SingleGeom &g, const float *filt, float *out, cudaStream_t stream, int band_h,
                   const DevInfo &dev, int min_band) {
-  auto kernel = k_conv2d_wide<K, K, FSRC, PF, GUARDS, HALO, L2D>;
+  auto kernel = k_conv2d_wide<K, K, FSRC, PF, GUARDS, HALO>;
   static OccCache occ_cache;
   const size_t ring = (PF >= 3) ? WideRing<K, (PF >= 3 ? PF : 2)>::kBytes : 0;
   SingleArgs a;
@@ -433,15 +433,6 @@ int launch_single(const SingleGeom &g, const float *filt, float *out, cudaStream
     case 27: if (constant_ok) return C2D_LW(FSRC_CONST, 2, 0); break;
     case 28: if (constant_ok) return C2D_LW(FSRC_CONST, 2, 2); break;
     case 29: return C2D_LW(FSRC_SMEM, 2, 0);
-    // L2 bulk prefetch of the row L2D ahead (prefetch_l2), on the default kernels' shapes
-    case 30: if (constant_ok) return launch_wide_v<K, FSRC_CONST, 1, 2, false, 4>(g, filt, out, stream, band_h, dev, min_band); break;
-    case 31: if (constant_ok) return launch_wide_v<K, FSRC_CONST, 1, 2, false, 8>(g, filt, out, stream, band_h, dev, min_band); break;
-    case 32: return launch_wide_v<K, FSRC_SMEM, 1, 0, false, 4>(g, filt, out, stream, band_h, dev, min_band);
-    case 33: if (constant_ok) return launch_single_v<K, 1, FSRC_CONST, 1, 1, false, 4>(g, filt, out, stream, band_h, dev, min_band); break;
-    case 34: if (constant_ok) return launch_single_v<K, 1, FSRC_CONST, 1, 1, false, 8>(g, filt, out, stream, band_h, dev, min_band); break;
-    case 35: if (constant_ok) return launch_single_v<K, 1, FSRC_CONST, 4, 1, false, 4>(g, filt, out, stream, band_h, dev, min_band); break;
-    case 36: if (constant_ok) return launch_single_v<K, 2, FSRC_CONST, 4, 0, false, 4>(g, filt, out, stream, band_h, dev, min_band); break;
-    case 37: if (constant_ok) return launch_single_v<K, 1, FSRC_CONST, 4, 2, false, 4>(g, filt, out, stream, band_h, dev, min_band); break;
     default: break;
   }
 #undef C2D_LW
