@@ -790,7 +790,7 @@ def cpu_baseline(workload, budget_s=10.0, batch=None):
     points, unit = workload_points(workload, batch)
     frac, _, _ = _calibrate(points, budget_s)
     u, s = _oracle_sample(points, frac)
-    what = "output rows" if points[0].kind == "single" else "images"
+    what = "output rows of the first image" if points[0].kind == "single" else "images"
     return {"value": round(u / s / 1e9, 6), "unit": unit, "cores": oracle.num_threads(), "kind": "oracle",
             "sample": f"first {frac * 100:.3g}% of the {what} of every point of the {workload} workload "
                       f"({s:.1f} s of oracle time; double accumulation, OpenMP over output rows)",
@@ -815,7 +815,7 @@ def run_reference(args):
         tot_u += u
         tot_s += s
     value = tot_u / tot_s / 1e9
-    what = "output rows" if points[0].kind == "single" else "images"
+    what = "output rows of the first image" if points[0].kind == "single" else "images"
     sample = (f"each step: first {frac * 100:.3g}% of the {what} of every point of the {args.workload} "
               f"workload (bounded sample; the full step would take ~{tot_s / args.steps / frac:.0f} s)")
     print(json.dumps({
