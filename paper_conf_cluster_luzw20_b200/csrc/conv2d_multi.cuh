@@ -35,30 +35,6 @@ struct Multi2Args {
   int aligned;
 };
 
-// Multi-channel filter slot of this unit's constant bank: the whole F x C x K x KP filter set of a call
-// (rows padded to KP floats), staged by the host like the single-channel slot (stream-ordered copy,
-// event-ordered reuse). 63 KiB: the bank also holds the single-channel slot.
-constexpr int kMultiConstFloats = 16128;
-__constant__ __align__(16) float c_mfilt[kMultiConstFloats];
-
-// filter row (fb, c, i) from the constant slot: filter f0 + fb, channel c, row i. With warp-uniform
-// control flow (one-warp CTAs) and a uniform f0 the compiler reads it with LDCU into uniform registers,
-// FFMA's UR operand: no shared-memory crossbar traffic (the bound of the shared-memory F-block, whose
-// broadcast LDS.128 moves 512 B for 4 values).
-template <int K, int FB>
-struct MultiFilterConst {
-  int f0, C;
-  __device__ __forceinline__ void row(float (&fr)[KCfg<K>::KP], int fb, int c, int i) const {
-    constexpr int KP = KCfg<K>::KP;
-    const float4 *p = reinterpret_cast<const float4 *>(c_mfilt + (((f0 + fb) * C + c) * K + i) * KP);
-#pragma unroll
-    for (int c4 = 0; c4 < KP / 4; ++c4) {
-      const float4 v = p[c4];
-      fr[4 * c4] = v.x; fr[4 * c4 + 1] = v.y; fr[4 * c4 + 2] = v.z; fr[4 * c4 + 3] = v.w;
-    }
-  }
-};
-
 // filter row (fb, c, i) of the CTA's F-block, staged in shared memory as [c][i][fb][KP]
 template <int K, int FB>
 struct MultiFilter {
@@ -288,45 +264,6 @@ __global__ void __launch_bounds__(kCtaWarps *kWarp, MINB) k_conv2d_multi2(const 
       multi_tile2<K, FB, U, SEG, GUARDS, PF, 1>(a, mf, n, seg_active, f0, x0, ob, oe, lane, ring_base);
   } else {
     multi_tile2<K, FB, U, SEG, GUARDS, PF, 2>(a, mf, n, seg_active, f0, x0, ob, oe, lane, ring_base);
-  }
-}
-
-// One-warp CTAs with the filter from the constant slot (MultiFilterConst). Tiles are ordered
-// ((fblk * n_groups + group) * n_bands + band) * n_cb + cb -- F-block-major, so the CTAs resident on the
-// GPU at any time share one or two F-blocks and the constant cache holds their filters (with the
-// image-major order of k_conv2d_multi2 every SM would touch every F-block: constant-cache thrash).
-// Every branch depends on blockIdx and kernel parameters only (uniform registers for the filter).
-template <int K, int FB, int SEG, int GUARDS, int PF, bool ALIGNED, int MINB>
-__global__ void __launch_bounds__(kWarp, MINB) k_conv2d_multic(const Multi2Args a) {
-  extern __shared__ __align__(16) float ring_smem_mc[];
-  const long long tile = blockIdx.x;
-  if (tile >= a.n_tiles) return;
-  const long long per_group = static_cast<long long>(a.n_cb) * a.n_bands;
-  const int cb = static_cast<int>(tile % a.n_cb);
-  const int band = static_cast<int>((tile / a.n_cb) % a.n_bands);
-  const int group = static_cast<int>((tile / per_group) % a.n_groups);
-  const int fblk = static_cast<int>(tile / (per_group * a.n_groups));
-  MultiFilterConst<K, FB> mf;
-  mf.f0 = fblk * FB;
-  mf.C = a.C;
-  const int lane = threadIdx.x;
-  const unsigned ring_base = static_cast<unsigned>(__cvta_generic_to_shared(ring_smem_mc));
-  const int ob = band * a.band_h;
-  if (ob >= a.Ho) return;
-  const int oe = min(ob + a.band_h, a.Ho);
-  const int x0 = cb * 4 * SEG;
-  constexpr int SEGS = kWarp / SEG;
-  const int n_raw = group * SEGS + lane / SEG;
-  const bool seg_active = n_raw < a.N;
-  const int n = seg_active ? n_raw : a.N - 1;
-  const bool inside = x0 + 4 * SEG + 4 * KCfg<K>::NE <= a.W;
-  if constexpr (ALIGNED) {
-    if (inside)
-      multi_tile2<K, FB, 1, SEG, GUARDS, PF, 0>(a, mf, n, seg_active, mf.f0, x0, ob, oe, lane, ring_base);
-    else
-      multi_tile2<K, FB, 1, SEG, GUARDS, PF, 1>(a, mf, n, seg_active, mf.f0, x0, ob, oe, lane, ring_base);
-  } else {
-    multi_tile2<K, FB, 1, SEG, GUARDS, PF, 2>(a, mf, n, seg_active, mf.f0, x0, ob, oe, lane, ring_base);
   }
 }
 

@@ -583,79 +583,6 @@ int launch_multi2_k(const float *in, int N, int C, int H, int W, const float *fi
   return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
 }
 
-// Multi-channel constant slot of this unit (c_mfilt), per device, recycled like g_cring.
-ConstRing g_mring[kMaxDevices];
-
-template <typename LaunchFn>
-int with_const_multi_filter(const float *filt, int rows, int K, int KP, cudaStream_t stream, const DevInfo &dev,
-                            LaunchFn launch) {
-  if (dev.id < 0 || dev.id >= kMaxDevices) return CONV2D_ECUDA;
-  ConstRing &ring = g_mring[dev.id];
-  std::lock_guard<std::mutex> lk(ring.mu);
-  if (!ring.init) {
-    void *p = nullptr;
-    if (cudaGetSymbolAddress(&p, c_mfilt) != cudaSuccess) return CONV2D_ECUDA;
-    ring.base = static_cast<float *>(p);
-    if (cudaEventCreateWithFlags(&ring.ev, cudaEventDisableTiming) != cudaSuccess) return CONV2D_ECUDA;
-    ring.init = true;
-  }
-  if (cudaStreamWaitEvent(stream, ring.ev, 0) != cudaSuccess) return CONV2D_ECUDA;
-  // F*C*K filter rows of K floats -> rows of KP floats
-  if (cudaMemcpy2DAsync(ring.base, KP * sizeof(float), filt, K * sizeof(float), K * sizeof(float), rows,
-                        cudaMemcpyDeviceToDevice, stream) != cudaSuccess)
-    return CONV2D_ECUDA;
-  const int rc = launch();
-  if (rc != CONV2D_OK) return rc;
-  if (cudaEventRecord(ring.ev, stream) != cudaSuccess) return CONV2D_ECUDA;
-  return CONV2D_OK;
-}
-
-// One-warp-CTA multi-channel kernel with the filter set in the constant slot (k_conv2d_multic). Returns
-// CONV2D_ESHAPE (caller falls back) when the padded filter set does not fit the slot.
-template <int K, int FB, int SEG, int GUARDS, int PF, int MINB>
-int launch_multic_v(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
-                    cudaStream_t stream, int band_h, const DevInfo &dev) {
-  constexpr int KP = KCfg<K>::KP;
-  constexpr int SEGS = kWarp / SEG;
-  const long long n_fb = (F + FB - 1) / FB;
-  if (n_fb * FB * C * K * KP > kMultiConstFloats) return CONV2D_ESHAPE;
-  const bool aligned = aligned16(in) && (W % 4 == 0);
-  Multi2Args a;
-  a.in = in;
-  a.filt = filt;
-  a.out = out;
-  a.N = N;
-  a.C = C;
-  a.H = H;
-  a.W = W;
-  a.F = F;
-  a.Ho = H - K + 1;
-  a.Wo = W - K + 1;
-  a.n_cb = ceil_div(a.Wo, 4 * SEG);
-  a.n_fb = static_cast<int>(n_fb);
-  a.n_groups = ceil_div(N, SEGS);
-  a.aligned = aligned ? 1 : 0;
-  const size_t ring = (PF >= 3) ? RowRing<K, 1, SEG, PF>::kBytes : 0;
-  auto go = [&](auto kernel, OccCache &occ_cache) {
-    // multi_bands counts 4-warp CTAs: resident one-warp CTAs / 4
-    const long long resident_warps =
-        static_cast<long long>(cta_occupancy(kernel, ring, occ_cache, kWarp)) * dev.num_sms;
-    int bh = band_h;
-    const int n_bands = multi_bands<K>(a.Ho, a.n_cb, static_cast<long long>(a.n_groups) * a.n_fb,
-                                       resident_warps / kCtaWarps > 0 ? resident_warps / kCtaWarps : 1, bh);
-    a.band_h = bh;
-    a.n_bands = n_bands;
-    a.n_tiles = static_cast<long long>(a.n_groups) * a.n_fb * n_bands * a.n_cb;
-    if (a.n_tiles > 0x7fffffffLL) return CONV2D_ESHAPE;
-    return with_const_multi_filter(filt, F * C * K, K, KP, stream, dev, [&]() {
-      kernel<<<static_cast<unsigned>(a.n_tiles), kWarp, ring, stream>>>(a);
-      return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
-    });
-  };
-  static OccCache occ_a, occ_m;
-  if (aligned) return go(k_conv2d_multic<K, FB, SEG, GUARDS, PF, true, MINB>, occ_a);
-  return go(k_conv2d_multic<K, FB, SEG, GUARDS, PF, false, 4>, occ_m);
-}
 
 template <int K, int FB, int U, int SEG, int GUARDS, int PF, int MINB = (SEG == kWarp && K <= 3 && FB * U >= 8) ? 2 : 3>
 int launch_multi2_v(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
@@ -709,20 +636,6 @@ int launch_multi(const float *in, int N, int C, int H, int W, const float *filt,
   if (mv == 70) return launch_multi2_v<K, FB, 1, 16, GUARDS, PF, 3>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
   if (mv == 71) return launch_multi2_v<K, FB, 1, 8, GUARDS, PF, 3>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
   if (mv == 72) return launch_multi2_v<K, FB, 1, 32, GUARDS, PF, 3>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
-  // constant-slot filter, one-warp CTAs, F-block-major tiles (k_conv2d_multic): FB x SEG
-  if (mv >= 80 && mv <= 87 && !stream_capturing(stream)) {
-    int r = CONV2D_ESHAPE;
-    switch (mv) {
-      case 80: r = launch_multic_v<K, FBH, 32, GUARDS, PF, 12>(in, N, C, H, W, filt, F, out, stream, band_h, dev); break;
-      case 81: r = launch_multic_v<K, FBH, 32, GUARDS, PF, 8>(in, N, C, H, W, filt, F, out, stream, band_h, dev); break;
-      case 82: r = launch_multic_v<K, FB, 32, GUARDS, PF, 8>(in, N, C, H, W, filt, F, out, stream, band_h, dev); break;
-      case 83: r = launch_multic_v<K, FB, 32, GUARDS, PF, 6>(in, N, C, H, W, filt, F, out, stream, band_h, dev); break;
-      case 84: r = launch_multic_v<K, FBH, 16, GUARDS, PF, 12>(in, N, C, H, W, filt, F, out, stream, band_h, dev); break;
-      case 85: r = launch_multic_v<K, FBH, 8, GUARDS, PF, 12>(in, N, C, H, W, filt, F, out, stream, band_h, dev); break;
-      default: break;
-    }
-    if (r != CONV2D_ESHAPE) return r;
-  }
 #undef C2D_LM2
 #endif
   // Tuned on B200 (tools/multi_variants.py): 16-lane segments (two images per warp) unless they waste
