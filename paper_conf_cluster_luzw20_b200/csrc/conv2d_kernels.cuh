@@ -320,19 +320,48 @@ __device__ __forceinline__ void store_row(float *__restrict__ orow, int x0, int 
 template <int K, int U, int FSRC, bool GUARD>
 __device__ __forceinline__ void row_step1(float (&acc)[K][U][4], const float (&w)[U][KCfg<K>::WN],
                                           const FilterSrc<K, FSRC> &fs, int qmin, int qmax) {
+  if constexpr (U == 2) {
+    // Paired FMA (sm_100 FFMA2, fma.rn.f32x2) across the two column chunks: one instruction runs the
+    // FMA chains of column v of chunk 0 and of chunk 1. Each component is an ordinary round-to-nearest
+    // fp32 FMA, so every output's sum is the same sequence of fmaf steps as the scalar chain -- the
+    // same bits -- but the FMA work takes half the issue slots (an FFMA2 = 64 FMAs occupies the FMA pipe
+    // for 2 cycles and leaves the other issue cycle to the shuffles, filter fetches, loads and stores;
+    // tools/ubench/ffma2_rate.cu: 99.8% of the fp32 peak vs 90-98% for FFMA). Every window value
+    // belongs to exactly one (chunk 0, chunk 1) pair, so forming the pairs costs no copies (pairs of
+    // adjacent columns (w[m], w[m+1]) straddle register pairs and cost ~200 MOVs per row at K=15); the
+    // broadcast filter value (f, f) is FFMA2's scalar uniform-register operand.
 #pragma unroll
-  for (int q = 0; q < K; ++q) {
-    if (!GUARD || (q >= qmin && q < qmax)) {
-      float fr[KCfg<K>::KP];
-      fs.row(fr, K - 1 - q);
-#pragma unroll
-      for (int u = 0; u < U; ++u) {
+    for (int q = 0; q < K; ++q) {
+      if (!GUARD || (q >= qmin && q < qmax)) {
+        float fr[KCfg<K>::KP];
+        fs.row(fr, K - 1 - q);
 #pragma unroll
         for (int v = 0; v < 4; ++v) {
-          float s = (q + 1 < K) ? acc[(q + 1 < K) ? q + 1 : 0][u][v] : 0.f;
+          float2 s = (q + 1 < K) ? make_float2(acc[(q + 1 < K) ? q + 1 : 0][0][v], acc[(q + 1 < K) ? q + 1 : 0][1][v])
+                                 : make_float2(0.f, 0.f);
 #pragma unroll
-          for (int j = 0; j < K; ++j) s = fmaf(w[u][v + j], fr[j], s);
-          acc[q][u][v] = s;
+          for (int j = 0; j < K; ++j)
+            s = __ffma2_rn(make_float2(w[0][v + j], w[1][v + j]), make_float2(fr[j], fr[j]), s);
+          acc[q][0][v] = s.x;
+          acc[q][1][v] = s.y;
+        }
+      }
+    }
+  } else {
+#pragma unroll
+    for (int q = 0; q < K; ++q) {
+      if (!GUARD || (q >= qmin && q < qmax)) {
+        float fr[KCfg<K>::KP];
+        fs.row(fr, K - 1 - q);
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+#pragma unroll
+          for (int v = 0; v < 4; ++v) {
+            float s = (q + 1 < K) ? acc[(q + 1 < K) ? q + 1 : 0][u][v] : 0.f;
+#pragma unroll
+            for (int j = 0; j < K; ++j) s = fmaf(w[u][v + j], fr[j], s);
+            acc[q][u][v] = s;
+          }
         }
       }
     }

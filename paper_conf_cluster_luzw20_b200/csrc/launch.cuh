@@ -417,6 +417,10 @@ int launch_single(const SingleGeom &g, const float *filt, float *out, cudaStream
     case 17: if (constant_ok) return C2D_LS(1, FSRC_CONST, 2, 0); break;
     case 18: if (constant_ok) return C2D_LS(2, FSRC_CONST, 2, 0); break;
     case 19: if (constant_ok) return C2D_LS(1, FSRC_CONST, 2, 2); break;
+    case 40: if (constant_ok) return C2D_LS(2, FSRC_CONST, 1, 1); break;
+    case 41: if (constant_ok) return C2D_LS(2, FSRC_CONST, 4, 1); break;
+    case 42: if (constant_ok) return C2D_LS(2, FSRC_CONST, 1, 2); break;
+    case 43: if (constant_ok) return C2D_LS(2, FSRC_CONST, 4, 2); break;
     default: break;
   }
 #undef C2D_LS

@@ -32,7 +32,7 @@ def main():
         pkg.conv2d_single(img((K + 40, 8200)), filt(K))          # wide image: constant slot, wide / ring kernels
         pkg.conv2d_single(img((K + 30, 1000)), filt(K))          # narrow: smem filter / split kernel (K >= 11)
         pkg.conv2d_single(img((K + 21, 517)), filt(K))           # ragged right edge
-        b = img((K * 300 + 7,))
+        b = img(((K + 20) * 300 + 4,))
         pkg.conv2d_single(b[1:1 + (K + 20) * 300].view(K + 20, 300), filt(K))  # misaligned rows
         pkg.conv2d_single_batch(img((3, K + 17, 700)), filt(K))
         pkg.conv2d_single_halo(img((40, 600)), img((K - 1, 600), 3), filt(K))
