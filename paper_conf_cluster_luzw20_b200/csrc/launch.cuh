@@ -374,13 +374,18 @@ int launch_single_default(const SingleGeom &g, const float *filt, float *out, cu
     if (W >= 8192) return C2D_LW(FSRC_CONST, 1, 2);
     return C2D_LS(1, FSRC_CONST, 4, 2);
   } else if constexpr (K <= 11) {
+    // two chunks with FFMA2 (row_step1) on images >= 4096 wide (profiles/r02l_ffma2*.txt: 8192^2 K=11
+    // x8 246 vs 231 Gpx/s)
+    if (W >= 4096) return C2D_LS(2, FSRC_CONST, 1, 2);
     return C2D_LS(1, FSRC_CONST, 4, 2);
   } else {
     // K = 12-14, wide: the cp.async ring with the guarded prologue (variant 15: 8192^2 K=13 155 -> 161
-    // Gpx/s, 4096^2 128 -> 132); K = 15 measured equal either way and keeps the register row fetch
+    // Gpx/s, 4096^2 128 -> 132); K = 15 measured equal either way and keeps the register row fetch.
+    // Two chunks with FFMA2 at 8192 (K <= 13: x8 178 vs 171) and below 4096 (2048^2 K=15 x8 98 vs 86).
+    if (K <= 13 && W >= 8192) return C2D_LS(2, FSRC_CONST, 1, 2);
     if (K <= 14 && W >= 4096) return C2D_LS(1, FSRC_CONST, 4, 1);
     if (W >= 4096) return C2D_LS(1, FSRC_CONST, 1, 1);
-    return C2D_LS(1, FSRC_CONST, 1, 2);
+    return C2D_LS(2, FSRC_CONST, 1, 2);
   }
 #undef C2D_LS
 #undef C2D_LW
