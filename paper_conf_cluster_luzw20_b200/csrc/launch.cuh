@@ -182,7 +182,7 @@ int launch_single_v(const SingleGeom &g, const float *filt, float *out, cudaStre
   constexpr int CTAW = (FSRC == FSRC_CONST) ? 1 : kCtaWarps;
   auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS, HALO>;
   static OccCache occ_cache;
-  const size_t ring = (PF >= 3) ? CTAW * RowRing<K, U, kWarp, (PF >= 3 ? PF : 2)>::kBytes : 0;
+  const size_t ring = (PF >= 3 && PF != 8) ? CTAW * RowRing<K, U, kWarp, (PF >= 3 ? PF : 2)>::kBytes : 0;
   SingleArgs a;
   fill_args(a, g, K, U, out);
   a.filt = filt;
@@ -208,7 +208,7 @@ int launch_wide_v(const SingleGeom &g, const float *filt, float *out, cudaStream
                   const DevInfo &dev, int min_band) {
   auto kernel = k_conv2d_wide<K, K, FSRC, PF, GUARDS, HALO>;
   static OccCache occ_cache;
-  const size_t ring = (PF >= 3) ? WideRing<K, (PF >= 3 ? PF : 2)>::kBytes : 0;
+  const size_t ring = (PF >= 3 && PF != 8) ? WideRing<K, (PF >= 3 ? PF : 2)>::kBytes : 0;
   SingleArgs a;
   fill_args(a, g, K, 2, out);  // n_cb in 256-column blocks (= two 128-column chunks)
   a.filt = filt;
@@ -426,6 +426,9 @@ int launch_single(const SingleGeom &g, const float *filt, float *out, cudaStream
     case 41: if (constant_ok) return C2D_LS(2, FSRC_CONST, 4, 1); break;
     case 42: if (constant_ok) return C2D_LS(2, FSRC_CONST, 1, 2); break;
     case 43: if (constant_ok) return C2D_LS(2, FSRC_CONST, 4, 2); break;
+    // ping-pong register prefetch (PF = 8), unrolled by two
+    case 44: if (constant_ok) return C2D_LS(1, FSRC_CONST, 8, 0); break;
+    case 45: if (constant_ok) return C2D_LS(2, FSRC_CONST, 8, 0); break;
     default: break;
   }
 #undef C2D_LS
@@ -442,6 +445,8 @@ int launch_single(const SingleGeom &g, const float *filt, float *out, cudaStream
     case 27: if (constant_ok) return C2D_LW(FSRC_CONST, 2, 0); break;
     case 28: if (constant_ok) return C2D_LW(FSRC_CONST, 2, 2); break;
     case 29: return C2D_LW(FSRC_SMEM, 2, 0);
+    case 46: if (constant_ok) return C2D_LW(FSRC_CONST, 8, 0); break;
+    case 47: return C2D_LW(FSRC_SMEM, 8, 0);
     default: break;
   }
 #undef C2D_LW
