@@ -427,7 +427,7 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const float *__
                                             float *__restrict__ outb, const FilterSrc<K, FSRC> &fs, int x0, int ob,
                                             int oe, int lane, unsigned ring_base) {
   constexpr bool SAFE = (EDGE != 0);
-  constexpr int NST = (PF >= 3 && PF != 8 && EDGE != 2) ? PF : 1;  // PF 8: ping-pong registers
+  constexpr int NST = (PF >= 3 && EDGE != 2) ? PF : 1;
   constexpr int RPF = (PF == 2 || (PF >= 3 && EDGE == 2)) ? ((PF == 2) ? 2 : 1) : 1;
   static_assert(NST == 1 || (NST & (NST - 1)) == 0, "ring depth must be a power of two");
   const int rend = oe + K - 1;  // input rows [ob, rend)
@@ -471,25 +471,6 @@ __device__ __forceinline__ void single_tile(const SingleArgs &a, const float *__
     return cur;
   };
   int r = ob;
-  if constexpr (PF == 8 && NST == 1) {
-    // ping-pong register prefetch, loop unrolled by two (see wide_tile): a buffer is refilled with row
-    // r+2 right after its window is built. All K slots every row (GUARDS ignored).
-    RowBuf<K, U> bA, bB;
-    load_row<K, U, SAFE>(bA, in_row<HALO>(a, inb, ob), x0, a.Wc, lane, a.aligned);
-    load_row<K, U, SAFE>(bB, in_row<HALO>(a, inb, min(ob + 1, rlast)), x0, a.Wc, lane, a.aligned);
-    auto body = [&](int rr, RowBuf<K, U> &buf) {
-      float w[U][KCfg<K>::WN];
-      build_windows<K, U>(buf, w, lane);
-      load_row<K, U, SAFE>(buf, in_row<HALO>(a, inb, min(rr + 2, rlast)), x0, a.Wc, lane, a.aligned);
-      row_step1<K, U, FSRC, false>(acc, w, fs, 0, K);
-      if (rr >= ob + K - 1) store_row<U, SAFE>(outb + static_cast<size_t>(rr - K + 1) * a.Po, x0, a.Wo, acc[0], lane);
-    };
-    for (; r < rend; r += 2) {
-      body(r, bA);
-      if (r + 1 < rend) body(r + 1, bB);
-    }
-    return;
-  }
   if constexpr (GUARDS == 0) {
     for (; r < rend; ++r) {
       const RowBuf<K, U> cur = next_row(r);

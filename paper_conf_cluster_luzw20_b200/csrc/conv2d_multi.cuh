@@ -49,6 +49,65 @@ struct MultiFilter {
   }
 };
 
+// The F-block staged as [c][i][j][fb] (filters fastest) for the paired-FMA step: one LDS.128 at (c, i, j)
+// returns the filter values of four consecutive filters, i.e. two aligned (fb, fb+1) register pairs.
+template <int K, int FB>
+struct MultiFilterP2 {
+  static_assert(FB % 2 == 0, "filter pairs");
+  unsigned sbase;
+  // fr2[p][j] = (w[f0+2p][c][i][j], w[f0+2p+1][c][i][j])
+  __device__ __forceinline__ void row2(float2 (&fr2)[FB / 2][K], int c, int i) const {
+#pragma unroll
+    for (int j = 0; j < K; ++j) {
+      const unsigned base = sbase + static_cast<unsigned>((((c * K + i) * K + j) * FB) * 4);
+      if constexpr (FB == 2) {
+        float x, y;
+        asm volatile("ld.shared.v2.f32 {%0, %1}, [%2];" : "=f"(x), "=f"(y) : "r"(base));
+        fr2[0][j] = make_float2(x, y);
+      } else {
+#pragma unroll
+        for (int p = 0; p < FB / 2; p += 2) {
+          float a0, a1, a2, a3;
+          lds4_at(base + p * 8, a0, a1, a2, a3);
+          fr2[p][j] = make_float2(a0, a1);
+          fr2[p + 1][j] = make_float2(a2, a3);
+        }
+      }
+    }
+  }
+};
+
+// a3 + a5 with paired FMA (sm_100 FFMA2): one instruction runs the chains of filters fb and fb+1 at the
+// same column -- the window value broadcast (FFMA2's scalar register operand), the filter pair from one
+// register pair, the accumulator pair. Same fmaf steps per output as row_step_multi: the same bits.
+template <int K, int FB, int U, bool SHIFT, bool GUARD>
+__device__ __forceinline__ void row_step_multi_p2(float (&acc)[K][FB][U][4], const float (&w)[U][KCfg<K>::WN],
+                                                  const MultiFilterP2<K, FB> &mf, int c, int qmin, int qmax) {
+#pragma unroll
+  for (int q = 0; q < K; ++q) {
+    if (!GUARD || (q >= qmin && q < qmax)) {
+      float2 fr2[FB / 2][K];
+      mf.row2(fr2, c, K - 1 - q);
+#pragma unroll
+      for (int p = 0; p < FB / 2; ++p) {
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+#pragma unroll
+          for (int v = 0; v < 4; ++v) {
+            const int qs = SHIFT ? ((q + 1 < K) ? q + 1 : 0) : q;
+            float2 s = (SHIFT && q + 1 >= K) ? make_float2(0.f, 0.f)
+                                              : make_float2(acc[qs][2 * p][u][v], acc[qs][2 * p + 1][u][v]);
+#pragma unroll
+            for (int j = 0; j < K; ++j) s = __ffma2_rn(make_float2(w[u][v + j], w[u][v + j]), fr2[p][j], s);
+            acc[q][2 * p][u][v] = s.x;
+            acc[q][2 * p + 1][u][v] = s.y;
+          }
+        }
+      }
+    }
+  }
+}
+
 // a3 + a5: one (row, channel) into the ring of FB filters x U chunks
 template <int K, int FB, int U, bool SHIFT, bool GUARD, typename MF>
 __device__ __forceinline__ void row_step_multi(float (&acc)[K][FB][U][4], const float (&w)[U][KCfg<K>::WN],
@@ -165,10 +224,17 @@ __device__ __forceinline__ void multi_tile2(const Multi2Args &a, const MF &mf, i
       advance();
       float w[U][KCfg<K>::WN];
       build_windows_g<K, U, SEG>(cur, w, lane);
-      if (c == 0)
-        row_step_multi<K, FB, U, true, G>(acc, w, mf, c, qmin, qmax);
-      else
-        row_step_multi<K, FB, U, false, G>(acc, w, mf, c, qmin, qmax);
+      if constexpr (std::is_same<MF, MultiFilterP2<K, FB>>::value) {
+        if (c == 0)
+          row_step_multi_p2<K, FB, U, true, G>(acc, w, mf, c, qmin, qmax);
+        else
+          row_step_multi_p2<K, FB, U, false, G>(acc, w, mf, c, qmin, qmax);
+      } else {
+        if (c == 0)
+          row_step_multi<K, FB, U, true, G>(acc, w, mf, c, qmin, qmax);
+        else
+          row_step_multi<K, FB, U, false, G>(acc, w, mf, c, qmin, qmax);
+      }
     }
   };
   auto store_slot0 = [&](int o) {
@@ -219,7 +285,8 @@ __device__ __forceinline__ void multi_tile2(const Multi2Args &a, const MF &mf, i
 // with W % 4 == 0 (interior + ragged-edge tiles); the misaligned case (guarded scalar loads) is its own
 // instantiation, so its register demand never caps -- or spills in -- the hot kernel (0 LDL/STL,
 // tests/test_sass.py).
-template <int K, int FB, int U, int SEG, int GUARDS, int PF, int MINB = 3, bool ALIGNED = true>
+// P2: paired FMA across filter pairs (row_step_multi_p2), F-block staged [c][i][j][fb].
+template <int K, int FB, int U, int SEG, int GUARDS, int PF, int MINB = 3, bool ALIGNED = true, bool P2 = false>
 __global__ void __launch_bounds__(kCtaWarps *kWarp, MINB) k_conv2d_multi2(const Multi2Args a) {
   constexpr int KP = KCfg<K>::KP;
   extern __shared__ __align__(16) float smem[];
@@ -227,17 +294,26 @@ __global__ void __launch_bounds__(kCtaWarps *kWarp, MINB) k_conv2d_multi2(const 
   const long long per_fb = static_cast<long long>(a.n_cb) * a.n_bands;
   const int fblk = static_cast<int>((tile0 / per_fb) % a.n_fb);
   const int f0 = fblk * FB;
-  const int total = a.C * K * FB * KP;
+  const int total = P2 ? a.C * K * K * FB : a.C * K * FB * KP;
   for (int t = threadIdx.x; t < total; t += blockDim.x) {
-    const int j = t % KP;
-    const int fb = (t / KP) % FB;
-    const int i = (t / (KP * FB)) % K;
-    const int c = t / (KP * FB * K);
+    int c, i, j, fb;
+    if constexpr (P2) {  // [c][i][j][fb]
+      fb = t % FB;
+      j = (t / FB) % K;
+      i = (t / (FB * K)) % K;
+      c = t / (FB * K * K);
+    } else {  // [c][i][fb][KP]
+      j = t % KP;
+      fb = (t / KP) % FB;
+      i = (t / (KP * FB)) % K;
+      c = t / (KP * FB * K);
+    }
     const int f = f0 + fb;
     smem[t] = (j < K && f < a.F) ? a.filt[((static_cast<size_t>(f) * a.C + c) * K + i) * K + j] : 0.f;
   }
   __syncthreads();
-  MultiFilter<K, FB> mf;
+  using MF = typename std::conditional<P2, MultiFilterP2<K, FB>, MultiFilter<K, FB>>::type;
+  MF mf;
   mf.sbase = static_cast<unsigned>(__cvta_generic_to_shared(smem));
   const int lane = threadIdx.x & (kWarp - 1);
   // this warp's cp.async row ring, after the F-block (16-byte aligned: total is a multiple of 4)

@@ -229,7 +229,7 @@ __device__ __forceinline__ void wide_tile(const SingleArgs &a, const float *__re
                                           const FilterRows<KH, KW, FSRC> &fs, int x0, int ob, int oe, int lane,
                                           unsigned ring_base) {
   constexpr bool SAFE = (EDGE != 0);
-  constexpr int NST = (PF >= 3 && PF != 8 && EDGE != 2) ? PF : 1;  // PF 8: ping-pong registers
+  constexpr int NST = (PF >= 3 && EDGE != 2) ? PF : 1;
   static_assert(NST == 1 || (NST & (NST - 1)) == 0, "ring depth must be a power of two");
   const int rend = oe + KH - 1;
   const int rlast = rend - 1;
@@ -272,28 +272,6 @@ __device__ __forceinline__ void wide_tile(const SingleArgs &a, const float *__re
   };
   auto out_at = [&](int o) { return outb + static_cast<size_t>(o) * a.Po; };
   int r = ob;
-  if constexpr (PF == 8 && NST == 1) {
-    // Ping-pong register prefetch, loop unrolled by two: rows alternate between two buffers, and a
-    // buffer is refilled (row r+2) right after its window is built, a whole iteration before it is
-    // read again. No register copies (PF 2's `n1 = n2`) and no copy of a still-loading register
-    // (PF 1's `cur = n1` waits on a load the compiler schedules late in the body: ncu long_scoreboard
-    // 41% of the stall samples at 8192^2 K=7). All K slots every row (GUARDS ignored).
-    WideRow bA, bB;
-    wide_load<KW, EDGE>(bA, in_row<HALO>(a, inb, ob), x0, a.Wc, lane);
-    wide_load<KW, EDGE>(bB, in_row<HALO>(a, inb, min(ob + 1, rlast)), x0, a.Wc, lane);
-    auto body = [&](int rr, WideRow &buf) {
-      float w[WideCfg<KW>::WN];
-      wide_window<KW>(buf, w, lane);
-      wide_load<KW, EDGE>(buf, in_row<HALO>(a, inb, min(rr + 2, rlast)), x0, a.Wc, lane);
-      wide_step<KH, KW, FSRC, false>(acc, w, fs, 0, KH);
-      if (rr >= ob + KH - 1) wide_store<SAFE>(out_at(rr - KH + 1), x0, a.Wo, acc[0], lane);
-    };
-    for (; r < rend; r += 2) {
-      body(r, bA);
-      if (r + 1 < rend) body(r + 1, bB);
-    }
-    return;
-  }
   if constexpr (GUARDS == 0) {
     for (; r < rend; ++r) {
       const WideRow cur = next_row(r);

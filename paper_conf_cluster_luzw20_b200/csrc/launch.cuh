@@ -182,7 +182,7 @@ int launch_single_v(const SingleGeom &g, const float *filt, float *out, cudaStre
   constexpr int CTAW = (FSRC == FSRC_CONST) ? 1 : kCtaWarps;
   auto kernel = k_conv2d_single<K, U, FSRC, CTAW, PF, GUARDS, HALO>;
   static OccCache occ_cache;
-  const size_t ring = (PF >= 3 && PF != 8) ? CTAW * RowRing<K, U, kWarp, (PF >= 3 ? PF : 2)>::kBytes : 0;
+  const size_t ring = (PF >= 3) ? CTAW * RowRing<K, U, kWarp, (PF >= 3 ? PF : 2)>::kBytes : 0;
   SingleArgs a;
   fill_args(a, g, K, U, out);
   a.filt = filt;
@@ -208,7 +208,7 @@ int launch_wide_v(const SingleGeom &g, const float *filt, float *out, cudaStream
                   const DevInfo &dev, int min_band) {
   auto kernel = k_conv2d_wide<K, K, FSRC, PF, GUARDS, HALO>;
   static OccCache occ_cache;
-  const size_t ring = (PF >= 3 && PF != 8) ? WideRing<K, (PF >= 3 ? PF : 2)>::kBytes : 0;
+  const size_t ring = (PF >= 3) ? WideRing<K, (PF >= 3 ? PF : 2)>::kBytes : 0;
   SingleArgs a;
   fill_args(a, g, K, 2, out);  // n_cb in 256-column blocks (= two 128-column chunks)
   a.filt = filt;
@@ -426,9 +426,6 @@ int launch_single(const SingleGeom &g, const float *filt, float *out, cudaStream
     case 41: if (constant_ok) return C2D_LS(2, FSRC_CONST, 4, 1); break;
     case 42: if (constant_ok) return C2D_LS(2, FSRC_CONST, 1, 2); break;
     case 43: if (constant_ok) return C2D_LS(2, FSRC_CONST, 4, 2); break;
-    // ping-pong register prefetch (PF = 8), unrolled by two
-    case 44: if (constant_ok) return C2D_LS(1, FSRC_CONST, 8, 0); break;
-    case 45: if (constant_ok) return C2D_LS(2, FSRC_CONST, 8, 0); break;
     default: break;
   }
 #undef C2D_LS
@@ -445,8 +442,6 @@ int launch_single(const SingleGeom &g, const float *filt, float *out, cudaStream
     case 27: if (constant_ok) return C2D_LW(FSRC_CONST, 2, 0); break;
     case 28: if (constant_ok) return C2D_LW(FSRC_CONST, 2, 2); break;
     case 29: return C2D_LW(FSRC_SMEM, 2, 0);
-    case 46: if (constant_ok) return C2D_LW(FSRC_CONST, 8, 0); break;
-    case 47: return C2D_LW(FSRC_SMEM, 8, 0);
     default: break;
   }
 #undef C2D_LW
@@ -559,16 +554,18 @@ int multi_bands(int Ho, int n_cb, long long groups, long long resident_ctas, int
   return n_bands;
 }
 
-template <int K, int FB, int U, int SEG, int GUARDS, int PF, int MINB, bool ALIGNED>
+template <int K, int FB, int U, int SEG, int GUARDS, int PF, int MINB, bool ALIGNED, bool P2 = false>
 int launch_multi2_k(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
                     cudaStream_t stream, int band_h, const DevInfo &dev) {
   constexpr int KP = KCfg<K>::KP;
   constexpr int SEGS = kWarp / SEG;
-  auto kernel = k_conv2d_multi2<K, FB, U, SEG, GUARDS, PF, MINB, ALIGNED>;
+  auto kernel = k_conv2d_multi2<K, FB, U, SEG, GUARDS, PF, MINB, ALIGNED, P2>;
   static OccCache occ_cache;
   static SmemOptIn smem_flag;
   const size_t ring = (PF >= 3) ? kCtaWarps * RowRing<K, U, SEG, PF>::kBytes : 0;
-  const size_t smem = static_cast<size_t>(C) * K * FB * KP * sizeof(float) + ring;
+  // F-block filters (+ 16 bytes: the P2 layout C*K*K*FB floats may leave the ring 8-byte aligned only)
+  const size_t fblock = P2 ? (static_cast<size_t>(C) * K * K * FB + 3) / 4 * 4 : static_cast<size_t>(C) * K * FB * KP;
+  const size_t smem = fblock * sizeof(float) + ring;
   if (int e = ensure_smem(kernel, smem, dev, smem_flag)) return e;
   Multi2Args a;
   a.in = in;
@@ -598,13 +595,15 @@ int launch_multi2_k(const float *in, int N, int C, int H, int W, const float *fi
 }
 
 
-template <int K, int FB, int U, int SEG, int GUARDS, int PF, int MINB = (SEG == kWarp && K <= 3 && FB * U >= 8) ? 2 : 3>
+template <int K, int FB, int U, int SEG, int GUARDS, int PF, int MINB = (SEG == kWarp && K <= 3 && FB * U >= 8) ? 2 : 3,
+          bool P2 = false>
 int launch_multi2_v(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
                     cudaStream_t stream, int band_h, const DevInfo &dev) {
   const bool aligned = aligned16(in) && (W % 4 == 0);
   if (!aligned)  // the misaligned-input instantiation (guarded scalar loads), its own register budget
-    return launch_multi2_k<K, FB, U, SEG, GUARDS, PF, 2, false>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
-  return launch_multi2_k<K, FB, U, SEG, GUARDS, PF, MINB, true>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
+    return launch_multi2_k<K, FB, U, SEG, GUARDS, PF, 2, false, P2>(in, N, C, H, W, filt, F, out, stream, band_h,
+                                                                    dev);
+  return launch_multi2_k<K, FB, U, SEG, GUARDS, PF, MINB, true, P2>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
 }
 
 
@@ -650,6 +649,13 @@ int launch_multi(const float *in, int N, int C, int H, int W, const float *filt,
   if (mv == 70) return launch_multi2_v<K, FB, 1, 16, GUARDS, PF, 3>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
   if (mv == 71) return launch_multi2_v<K, FB, 1, 8, GUARDS, PF, 3>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
   if (mv == 72) return launch_multi2_v<K, FB, 1, 32, GUARDS, PF, 3>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
+  // paired FMA across filter pairs (row_step_multi_p2), the default FB: 16 / 8 / 32 lanes
+  if constexpr (FBD % 2 == 0) {
+    if (mv == 90) return launch_multi2_v<K, FBD, 1, 16, GUARDS, PF, 3, true>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
+    if (mv == 91) return launch_multi2_v<K, FBD, 1, 8, GUARDS, PF, 3, true>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
+    if (mv == 92) return launch_multi2_v<K, FBD, 1, 32, GUARDS, PF, 2, true>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
+    if (mv == 93) return launch_multi2_v<K, FBD, 1, 16, GUARDS, PF, 2, true>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
+  }
 #undef C2D_LM2
 #endif
   // Tuned on B200 (tools/multi_variants.py): 16-lane segments (two images per warp) unless they waste
