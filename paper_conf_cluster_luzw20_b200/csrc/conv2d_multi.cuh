@@ -316,8 +316,9 @@ __global__ void __launch_bounds__(kCtaWarps *kWarp, MINB) k_conv2d_multi2(const 
   MF mf;
   mf.sbase = static_cast<unsigned>(__cvta_generic_to_shared(smem));
   const int lane = threadIdx.x & (kWarp - 1);
-  // this warp's cp.async row ring, after the F-block (16-byte aligned: total is a multiple of 4)
-  const unsigned ring_base = mf.sbase + static_cast<unsigned>(total) * 4u +
+  // this warp's cp.async row ring, after the F-block, 16-byte aligned (the P2 layout C*K*K*FB may not be a
+  // multiple of 4 floats)
+  const unsigned ring_base = mf.sbase + static_cast<unsigned>((total + 3) / 4 * 4) * 4u +
                              (threadIdx.x >> 5) * RowRing<K, U, SEG, (PF >= 3 ? PF : 2)>::kBytes;
   const long long tile = tile0 + (threadIdx.x >> 5);
   if (tile >= a.n_tiles) return;
