@@ -665,10 +665,18 @@ int launch_multi(const float *in, int N, int C, int H, int W, const float *filt,
   // 8-lane segments (four images per warp, 32 columns each) for narrow layers: Table I's 8-26-column
   // outputs use 25-81% of the lanes instead of 12-41% (tools/multi_band_sweep.py)
   const bool seg8 = mv == 0 && N >= 4 && Wo <= 32 && lane_use(Wo, 32) >= lane_use(Wo, 64) + 0.15;
+  // K = 4..7 (two filters per warp): paired FMA across the filter pair (row_step_multi_p2, FFMA2) --
+  // profiles/r02p_multi_p2.txt: configs[3] 42.6 vs 37.6 TFLOP/s, Table I K=5 layers +5-20%. K <= 3 (eight
+  // filters per warp) keeps the scalar FMAs: its FFMA2 form spills at 3 CTAs per SM and loses at 2.
+  constexpr bool P2 = (K >= 4 && K <= 7 && FBD % 2 == 0);
+#define C2D_LMP(SEGG) \
+  launch_multi2_v<K, FBD, 1, SEGG, GUARDS, PF, (SEGG == kWarp && K <= 3 && FBD >= 8) ? 2 : 3, P2>( \
+      in, N, C, H, W, filt, F, out, stream, band_h, dev)
   if (seg8)
-    rc = C2D_LM(FBD, 8);
+    rc = C2D_LMP(8);
   else
-    rc = seg16 ? C2D_LM(FBD, 16) : C2D_LM(FBD, 32);
+    rc = seg16 ? C2D_LMP(16) : C2D_LMP(32);
+#undef C2D_LMP
 #undef C2D_LM
   if (rc != CONV2D_ESHAPE) return rc;
   // F-block does not fit shared memory: round-1 kernel with one filter per warp
