@@ -351,16 +351,27 @@ int launch_single_default(const SingleGeom &g, const float *filt, float *out, cu
   // Small images with K < 11 are latency-bound (a few microseconds): the per-CTA shared-memory filter
   // skips the constant-slot staging (a stream-ordered copy plus two event operations, ~3 us of host
   // and device time per call, tools/host_overhead.py). Same summation order, same bits.
-  const long long px = static_cast<long long>(g.H) * W * g.N;
+  const long long px = static_cast<long long>(g.H) * W * g.N;  // input pixels of the launch (all images)
   const bool small = px <= 512LL * 512 || (K <= 5 && px <= 1024LL * 1024);
+  // Launches with >= 32 M (128 M) input pixels amortise the constant-slot staging (a stream-ordered copy
+  // + event ops, ~3 us) and take the constant-filter kernels that win on long launches; shorter ones
+  // keep the per-CTA shared-memory filter (profiles/r02q_all_b8.txt: batches of 8; r02c/r02e/r02l: one
+  // image).
+  const bool big = px >= (32LL << 20), giant = px >= (128LL << 20);
+  const bool cst = constant_ok && !force_smem;
   if constexpr (K <= 3) {
-    if (constant_ok && !force_smem && W >= 8192) return C2D_LW(FSRC_CONST, 1, 2);
+    // wide lanes; constant slot on long launches (4096^2 x8 686 vs 642 Gpx/s), shared memory otherwise
+    // (one 4096^2 image 511 vs 442)
+    if (cst && W >= 4096 && big) return C2D_LW(FSRC_CONST, 1, 0);
     return C2D_LW(FSRC_SMEM, 1, 0);
   }
   if constexpr (K <= 5) {
-    if (!constant_ok || force_smem || W <= 2048) return C2D_LW(FSRC_SMEM, 1, 0);
+    // two chunks (FFMA2) + ring + guards on launches >= 16 M pixels (x8: 8192^2 711 vs 649, 2048^2 536 vs
+    // 466; one 4096^2 image 467 vs 419), wide lanes + shared memory below (one 2048^2 image 227 vs 217)
+    if (cst && px >= (16LL << 20) && W >= 2048) return C2D_LS(2, FSRC_CONST, 4, 2);
+    if (!cst || W <= 2048) return C2D_LW(FSRC_SMEM, 1, 0);
   }
-  if (!constant_ok || force_smem || (K < 11 && small)) {
+  if (!cst || (K < 11 && small)) {
     if constexpr (K <= 7) return C2D_LS(2, FSRC_SMEM, 1, 0);
     else return C2D_LS(1, FSRC_SMEM, 1, 0);
   }
@@ -368,9 +379,11 @@ int launch_single_default(const SingleGeom &g, const float *filt, float *out, cu
     return C2D_LS(2, FSRC_CONST, 4, 0);
   } else if constexpr (K <= 7) {
     if (W >= 8192) return C2D_LW(FSRC_CONST, 1, 2);
+    if (big) return C2D_LW(FSRC_CONST, 1, 0);  // x8: 4096^2 486 vs 449, 2048^2 402 vs 374
     if (W >= 4096) return C2D_LS(2, FSRC_CONST, 4, 2);
     return C2D_LS(1, FSRC_CONST, 4, 2);
   } else if constexpr (K <= 9) {
+    if (W >= 8192 && giant) return C2D_LS(2, FSRC_CONST, 1, 0);  // x8 349 vs 338 (one image: -11%)
     if (W >= 8192) return C2D_LW(FSRC_CONST, 1, 2);
     return C2D_LS(1, FSRC_CONST, 4, 2);
   } else if constexpr (K <= 11) {
@@ -381,10 +394,12 @@ int launch_single_default(const SingleGeom &g, const float *filt, float *out, cu
   } else {
     // K = 12-14, wide: the cp.async ring with the guarded prologue (variant 15: 8192^2 K=13 155 -> 161
     // Gpx/s, 4096^2 128 -> 132); K = 15 measured equal either way and keeps the register row fetch.
-    // Two chunks with FFMA2 at 8192 (K <= 13: x8 178 vs 171) and below 4096 (2048^2 K=15 x8 98 vs 86).
+    // Two chunks with FFMA2 at 8192 (K <= 13: x8 178 vs 171); below 4096 two chunks for short launches,
+    // the one-chunk ring on long ones (2048^2 K=15 x8 107 vs 101).
     if (K <= 13 && W >= 8192) return C2D_LS(2, FSRC_CONST, 1, 2);
     if (K <= 14 && W >= 4096) return C2D_LS(1, FSRC_CONST, 4, 1);
     if (W >= 4096) return C2D_LS(1, FSRC_CONST, 1, 1);
+    if (big) return C2D_LS(1, FSRC_CONST, 4, 1);
     return C2D_LS(2, FSRC_CONST, 1, 2);
   }
 #undef C2D_LS
