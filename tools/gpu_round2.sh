@@ -49,4 +49,5 @@ prof prof_conv11c1 k_conv2d_multi multi 128,1,224,224,64 3
 prof prof_multi_config3 k_conv2d_multi multi 128,3,224,224,64 7
 prof prof_tc_config2 k_conv2d_multi_tc multi 32,64,56,56,64 3 --tc
 prof prof_tc_config3 k_conv2d_multi_tc multi 128,3,224,224,64 7 --tc
+prof prof_config0 "k_conv2d_(single|wide)" single 256 3
 ls -la gpurun_out | tail -40

@@ -37,6 +37,7 @@ CAPTURES = {
     "prof_multi_config3": "conv2d_multi N128 C3 F64 224^2 K7",
     "prof_split_k15_s1024": "conv2d_single 1024^2 K=15 (filter-row split, cluster of 2 CTAs)",
     "prof_conv11c1": "conv2d_multi Table I CONV11 C1 N128 224^2 F64 K3",
+    "prof_config0": "conv2d_single 256^2 K=3 (configs[0], one image)",
 }
 
 
