@@ -15,6 +15,7 @@
 #include "conv2d_multi.cuh"
 #include "conv2d_split.cuh"
 #include "conv2d_wide.cuh"
+#include "conv2d_pair.cuh"
 
 namespace {
 
@@ -223,6 +224,56 @@ int launch_wide_v(const SingleGeom &g, const float *filt, float *out, cudaStream
   };
   if constexpr (FSRC == FSRC_CONST) return with_const_filter(filt, K, KCfg<K>::KP, stream, dev, go);
   return go();
+}
+
+// Slot-paired FFMA2 kernel (conv2d_pair.cuh), odd K: the constant slot holds the pair table
+//   pairs [p][j] = (f[H+p][j], f[p][j]), single [j] = f[H-1][j]
+// built by three stream-ordered copies (two interleave 4-byte elements at an 8-byte destination pitch),
+// recycled with the slot's event like the plain filter staging.
+template <int K, typename LaunchFn>
+int with_const_pair_filter(const float *filt, cudaStream_t stream, const DevInfo &dev, LaunchFn launch) {
+  using PC = PairCfg<K>;
+  if (dev.id < 0 || dev.id >= kMaxDevices) return CONV2D_ECUDA;
+  ConstRing &ring = g_cring[dev.id];
+  std::lock_guard<std::mutex> lk(ring.mu);
+  if (!ring.init) {
+    void *p = nullptr;
+    if (cudaGetSymbolAddress(&p, c_filt) != cudaSuccess) return CONV2D_ECUDA;
+    ring.base = static_cast<float *>(p);
+    if (cudaEventCreateWithFlags(&ring.ev, cudaEventDisableTiming) != cudaSuccess) return CONV2D_ECUDA;
+    ring.init = true;
+  }
+  if (cudaStreamWaitEvent(stream, ring.ev, 0) != cudaSuccess) return CONV2D_ECUDA;
+  const size_t n = static_cast<size_t>(PC::NP) * K;
+  if (cudaMemcpy2DAsync(ring.base, 8, filt + PC::H * K, 4, 4, n, cudaMemcpyDeviceToDevice, stream) != cudaSuccess ||
+      cudaMemcpy2DAsync(ring.base + 1, 8, filt, 4, 4, n, cudaMemcpyDeviceToDevice, stream) != cudaSuccess ||
+      cudaMemcpyAsync(ring.base + PC::kSingle, filt + (PC::H - 1) * K, K * sizeof(float), cudaMemcpyDeviceToDevice,
+                      stream) != cudaSuccess)
+    return CONV2D_ECUDA;
+  const int rc = launch();
+  if (rc != CONV2D_OK) return rc;
+  if (cudaEventRecord(ring.ev, stream) != cudaSuccess) return CONV2D_ECUDA;
+  return CONV2D_OK;
+}
+
+template <int K, int PF, bool HALO = false>
+int launch_pair_v(const SingleGeom &g, const float *filt, float *out, cudaStream_t stream, int band_h,
+                  const DevInfo &dev, int min_band) {
+  auto kernel = k_conv2d_pair<K, PF, HALO>;
+  static OccCache occ_cache;
+  const size_t ring = (PF >= 3) ? RowRing<K, 1, kWarp, (PF >= 3 ? PF : 2)>::kBytes : 0;
+  SingleArgs a;
+  fill_args(a, g, K, 1, out);
+  a.filt = filt;
+  const long long resident = static_cast<long long>(cta_occupancy(kernel, ring, occ_cache, kWarp)) * dev.num_sms;
+  a.n_bands = band_count(a.Ho, K, a.n_cb, a.n_img, resident, band_h, min_band);
+  const long long tiles = static_cast<long long>(a.n_cb) * a.n_bands * a.n_img;
+  if (tiles > 0x7fffffffLL) return CONV2D_ESHAPE;
+  a.n_tiles = static_cast<int>(tiles);
+  return with_const_pair_filter<K>(filt, stream, dev, [&]() {
+    kernel<<<a.n_tiles, kWarp, ring, stream>>>(a);
+    return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
+  });
 }
 
 // Rectangular KH x KW filters (conv2d_single_rect): the wide-lane kernel with a KH-slot
@@ -441,6 +492,9 @@ int launch_single(const SingleGeom &g, const float *filt, float *out, cudaStream
     case 41: if (constant_ok) return C2D_LS(2, FSRC_CONST, 4, 1); break;
     case 42: if (constant_ok) return C2D_LS(2, FSRC_CONST, 1, 2); break;
     case 43: if (constant_ok) return C2D_LS(2, FSRC_CONST, 4, 2); break;
+    // slot-paired FFMA2 ring (conv2d_pair.cuh), odd K
+    case 48: if constexpr (K % 2 == 1 && K >= 3) { if (constant_ok) return launch_pair_v<K, 1>(g, filt, out, stream, band_h, dev, min_band); } break;
+    case 49: if constexpr (K % 2 == 1 && K >= 3) { if (constant_ok) return launch_pair_v<K, 4>(g, filt, out, stream, band_h, dev, min_band); } break;
     default: break;
   }
 #undef C2D_LS
