@@ -429,6 +429,10 @@ int launch_single_default(const SingleGeom &g, const float *filt, float *out, cu
   if constexpr (K <= 5) {
     return C2D_LS(2, FSRC_CONST, 4, 0);
   } else if constexpr (K <= 7) {
+    // slot-paired FFMA2 ring on the longest launches (r02r: 8 x 8192^2 K=7 528 vs 511 Gpx/s)
+    if constexpr (K == 7) {
+      if (W >= 8192 && giant) return launch_pair_v<K, 4, HALO>(g, filt, out, stream, band_h, dev, min_band);
+    }
     if (W >= 8192) return C2D_LW(FSRC_CONST, 1, 2);
     if (big) return C2D_LW(FSRC_CONST, 1, 0);  // x8: 4096^2 486 vs 449, 2048^2 402 vs 374
     if (W >= 4096) return C2D_LS(2, FSRC_CONST, 4, 2);
@@ -447,6 +451,11 @@ int launch_single_default(const SingleGeom &g, const float *filt, float *out, cu
     // Gpx/s, 4096^2 128 -> 132); K = 15 measured equal either way and keeps the register row fetch.
     // Two chunks with FFMA2 at 8192 (K <= 13: x8 178 vs 171); below 4096 two chunks for short launches,
     // the one-chunk ring on long ones (2048^2 K=15 x8 107 vs 101).
+    // K = 15 on long launches >= 4096 wide: the slot-paired FFMA2 ring (conv2d_pair.cuh; r02r: 8 x 8192^2
+    // 132 vs 124 Gpx/s, 8 x 4096^2 125 vs 118, one 8192^2 image 122 vs 117)
+    if constexpr (K == 15) {
+      if (W >= 4096 && big) return launch_pair_v<K, 4, HALO>(g, filt, out, stream, band_h, dev, min_band);
+    }
     if (K <= 13 && W >= 8192) return C2D_LS(2, FSRC_CONST, 1, 2);
     if (K <= 14 && W >= 4096) return C2D_LS(1, FSRC_CONST, 4, 1);
     if (W >= 4096) return C2D_LS(1, FSRC_CONST, 1, 1);
