@@ -180,11 +180,12 @@ def test_config4_32768_k15_seams_and_bands(cuda_device):
             assert torch.equal(part, y[a0:a1]), (b.rank, a0, a1)
 
 
-@pytest.mark.parametrize("variant", [1, 2, 3, 4, 5, 6, 7, 9, 13, 15])
+@pytest.mark.parametrize("variant", [1, 2, 3, 4, 5, 6, 7, 9, 13, 15, 20, 22, 23, 25, 26, 27, 40, 42, 43, 48, 49])
 def test_every_kernel_variant_bitwise_equal(cuda_device, variant):
-    """Every instantiation (filter in shared / constant memory, 1 or 2 column chunks, guarded or
-    unguarded band prologue/epilogue) of the one-warp-tile kernel gives the same bits as variant 1,
-    and passes the oracle. (The default takes the filter-row split kernel for W <= 1024, K >= 11;
+    """Every instantiation (filter in shared / constant memory, 1 or 2 column chunks -- the two-chunk
+    ones with FFMA2 --, guarded or unguarded band prologue/epilogue, wide lanes 20-29, the slot-paired
+    FFMA2 ring 48/49) of the one-warp-tile kernels gives the same bits as variant 1, and passes the
+    oracle. (The default takes the filter-row split kernel for W <= 1024, K >= 11;
     its bits are covered by test_split_variants.)"""
     shapes = [(40, 300), (77, 1030), (300, 517)]
     try:
