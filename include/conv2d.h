@@ -73,9 +73,13 @@ int conv2d_single(const float *in, int H, int W, const float *filt, int K, float
  *   filt : F*C*K*K floats (FCKK == torch OIHW)
  *   out  : N*F*(H-K+1)*(W-K+1) floats (NFHoWo):
  *          out[n][f][y][x] = sum_{c<C} sum_{i<K} sum_{j<K} in[n][c][y+i][x+j] * filt[f][c][i][j]
- *   The filters of one F-block (all C channels) are staged in shared memory; the F-block shrinks to
- *   one filter when needed, so C*K*ceil(K/4)*4*4 bytes must fit in a CTA's shared memory (227 KiB:
- *   e.g. C <= 236 at K = 15, C <= 4843 at K = 3); larger C returns CONV2D_ESHAPE.
+ *   Kernel: the filter-blocked wide-lane kernel (a lane owns 8 output columns x FB = 8 or 4 filters;
+ *   column reuse by warp shuffle). Each output sums its C*K*K terms in
+ *   (filter row i, channel c, filter column j) order, one fmaf chain -- exact on integer data,
+ *   independent of batch, tiling and F-block. The filters of one F-block (all C channels) are staged
+ *   in shared memory (C*K*K*FB*4 bytes); when even FB = 4 does not fit, the round-1 kernel with one
+ *   filter per warp takes over (C*K*ceil(K/4)*4*4 bytes: e.g. C <= 236 at K = 15, C <= 4843 at
+ *   K = 3); larger C returns CONV2D_ESHAPE.
  */
 int conv2d_multi(const float *in, int N, int C, int H, int W, const float *filt, int F, int K,
                  float *out, void *stream);
@@ -104,10 +108,11 @@ int conv2d_single_rect(const float *in, int H, int W, const float *filt, int FH,
                        void *stream);
 
 /*
- * Same as conv2d_single / conv2d_multi with an explicit output-row band height per warp
- * (band_h <= 0: the library's choice). For tuning sweeps and tests of the band / halo logic; the
- * result is bitwise identical for every band_h (each output's summation order does not depend on
- * its band).
+ * Same as conv2d_single / conv2d_multi with an explicit tiling parameter (band_h <= 0: the library's
+ * choice): conv2d_single_ex -- the output-row band height per warp; conv2d_multi_ex -- the warp-steps
+ * per warp of the filter-blocked kernel (a warp-step = 32/SEG output-row segments). For tuning sweeps
+ * and tests of the band / halo logic; the result is bitwise identical for every band_h (each
+ * output's summation order does not depend on its tile).
  */
 int conv2d_single_ex(const float *in, int H, int W, const float *filt, int K, float *out, void *stream,
                      int band_h);

@@ -16,6 +16,7 @@
 #include "conv2d_split.cuh"
 #include "conv2d_wide.cuh"
 #include "conv2d_pair.cuh"
+#include "conv2d_mob.cuh"
 
 namespace {
 
@@ -685,6 +686,138 @@ int launch_multi2_v(const float *in, int N, int C, int H, int W, const float *fi
 }
 
 
+// Filter-blocked multi-channel kernel (conv2d_mob.cuh). Warp-steps per warp L: the grid runs
+// ceil(ctas / resident) waves of L steps each, so pick L minimising waves(L) * (L + 0.05) (the 0.05 step
+// of F-block staging per CTA breaks ties towards fewer, longer CTAs). Returns CONV2D_ESHAPE when the
+// F-block does not fit shared memory.
+template <int K, int FB, int SEG, int EDGE, int MINB, bool PFL1 = false>
+int launch_mob_k(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
+                 cudaStream_t stream, int L_req, const DevInfo &dev, long long *plan = nullptr) {
+  constexpr int SEGS = kWarp / SEG;
+  auto kernel = k_conv2d_mob<K, FB, SEG, EDGE, MINB, PFL1>;
+  static OccCache occ_cache;
+  static SmemOptIn smem_flag;
+  const size_t smem = static_cast<size_t>(C) * K * K * FB * sizeof(float);
+  if (int e = ensure_smem(kernel, smem, dev, smem_flag)) return e;
+  MobArgs a;
+  a.in = in;
+  a.filt = filt;
+  a.out = out;
+  a.N = N;
+  a.C = C;
+  a.H = H;
+  a.W = W;
+  a.F = F;
+  a.Ho = H - K + 1;
+  a.Wo = W - K + 1;
+  a.n_cb = ceil_div(a.Wo, kWideV * SEG);
+  const long long units = static_cast<long long>(N) * a.Ho * a.n_cb;
+  // 32-bit unit indices and channel-plane offsets in the kernel
+  if (units + kCtaWarps * SEGS >= 0x7fffffffLL || static_cast<long long>(N) * C * H * W >= 0x7fffffffLL)
+    return CONV2D_ESHAPE;  // (the round-1 kernel takes such tensors)
+  a.units_img = a.Ho * a.n_cb;
+  a.units = static_cast<int>(units);
+  a.steps = (a.units + SEGS - 1) / SEGS;
+  const int n_fb = ceil_div(F, FB);
+  const uintptr_t ob = reinterpret_cast<uintptr_t>(out);
+  a.ovec = ((ob & 15u) == 0 && a.Wo % 4 == 0) ? 2 : (((ob & 7u) == 0 && a.Wo % 2 == 0) ? 1 : 0);
+  int L = L_req;
+  const long long resident =
+      static_cast<long long>(cta_occupancy(kernel, smem, occ_cache, kCtaWarps * kWarp)) * dev.num_sms;
+  if (L <= 0) {
+    const long long lmax = (a.steps + kCtaWarps - 1) / kCtaWarps;
+    double best = 1e300;
+    L = 1;
+    for (long long l = 1; l <= lmax; ++l) {
+      const long long ctas = static_cast<long long>(n_fb) * ((a.steps + kCtaWarps * l - 1) / (kCtaWarps * l));
+      const long long waves = (ctas + resident - 1) / resident;
+      const double cost = static_cast<double>(waves) * (static_cast<double>(l) + 0.05);
+      if (cost < best - 1e-9) {
+        best = cost;
+        L = static_cast<int>(l);
+      }
+    }
+  }
+  a.L = L;
+  a.n_fb = n_fb;
+  a.ctas_fb = static_cast<int>((a.steps + static_cast<long long>(kCtaWarps) * L - 1) / (static_cast<long long>(kCtaWarps) * L));
+  const long long blocks = static_cast<long long>(n_fb) * a.ctas_fb;
+  if (blocks > 0x7fffffffLL) return CONV2D_ESHAPE;
+  if (plan) {  // dry run: grid size and resident CTAs per wave
+    plan[0] = blocks;
+    plan[1] = resident;
+    return CONV2D_OK;
+  }
+  kernel<<<static_cast<unsigned>(blocks), kCtaWarps * kWarp, smem, stream>>>(a);
+  return cudaGetLastError() == cudaSuccess ? CONV2D_OK : CONV2D_ECUDA;
+}
+
+// segment width (lanes) of the filter-blocked kernel: the most lanes on valid columns (8*SEG-column
+// units; a unit never straddles rows), ties to the wider segment. 32-lane segments are never strictly
+// better than 16 (two 128-column units cover any row a 256-column unit covers) and are left to the
+// tuning build.
+inline int mob_seg(int Wo) {
+  int best = 16;
+  double bu = -1.0;
+  for (int seg = 16; seg >= 4; seg /= 2) {
+    const int span = kWideV * seg;
+    const double u = double(Wo) / (double((Wo + span - 1) / span) * span);
+    if (u > bu + 1e-9) {
+      bu = u;
+      best = seg;
+    }
+  }
+  return best;
+}
+
+// aligned rows (W % 4 == 0, 16-byte base): clamped vector loads at MINB CTAs per SM; misaligned rows:
+// the guarded scalar-load instantiation at MINB2 (its own register budget: 0 spills)
+template <int K, int FB, int MINB, bool PFL1 = false, int MINB2 = (FB == 8 ? 2 : 3)>
+int launch_mob(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
+               cudaStream_t stream, int seg, int L_req, const DevInfo &dev, long long *plan = nullptr) {
+  const bool aligned = aligned16(in) && (W % 4 == 0);
+  if (seg <= 0) seg = mob_seg(W - K + 1);
+#define C2D_MOB(S)                                                                                                \
+  case S:                                                                                                         \
+    return aligned ? launch_mob_k<K, FB, S, 1, MINB, PFL1>(in, N, C, H, W, filt, F, out, stream, L_req, dev, plan) \
+                   : launch_mob_k<K, FB, S, 2, MINB2>(in, N, C, H, W, filt, F, out, stream, L_req, dev, plan);
+  switch (seg) {
+    C2D_MOB(4) C2D_MOB(8) C2D_MOB(16)
+#ifdef C2D_TUNING
+    C2D_MOB(32)
+#endif
+    default: return CONV2D_ESHAPE;
+  }
+#undef C2D_MOB
+}
+
+// The product multi-channel path (conv2d_mob.cuh). FB = 8 filters per lane at 3 CTAs per SM (168
+// registers) for K <= 8 except K = 5, unless its grid fills less than 3/4 of one wave -- then FB = 4
+// (twice the CTAs, 4 CTAs per SM up to K = 6): Table I CONV4/6/7, tools/multi_variants.py,
+// profiles/r02_mob*. K = 5 and K >= 9: FB = 4 (ptxas spills FB = 8 there at 168 registers; 0 LDL/STL
+// in every product kernel, tests/test_sass.py). band_h > 0: warp-steps per warp (explicit tiling;
+// same bits). Returns CONV2D_ESHAPE when the F-block does not fit shared memory (caller falls back).
+template <int K>
+int launch_mob_auto(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
+                    cudaStream_t stream, int band_h, const DevInfo &dev) {
+  constexpr int M4 = (K <= 6) ? 4 : 3;
+  const int L = band_h > 0 ? band_h : 0;
+  if constexpr (K <= 8 && K != 5) {
+    long long plan[2] = {0, 0};
+    const int e = launch_mob<K, 8, 3>(in, N, C, H, W, filt, F, out, stream, 0, L, dev, plan);
+    if (e == CONV2D_OK && 4 * plan[0] >= 3 * plan[1]) {
+      // K <= 4 with several channels: rows carry few FMAs and L1 misses (a new channel plane every
+      // row) are exposed at one row of register prefetch -- an L1 prefetch two rows ahead: configs[2]
+      // 25.6 -> 29.9 TFLOP/s, Table I C=3 K=3 layers +5-17%; C = 1 and K = 7 lose (profiles/r02_mob*)
+      if constexpr (K <= 4)
+        if (C >= 2) return launch_mob<K, 8, 3, true>(in, N, C, H, W, filt, F, out, stream, 0, L, dev);
+      return launch_mob<K, 8, 3>(in, N, C, H, W, filt, F, out, stream, 0, L, dev);
+    }
+    if (e != CONV2D_OK && e != CONV2D_ESHAPE) return e;
+  }
+  return launch_mob<K, 4, M4>(in, N, C, H, W, filt, F, out, stream, 0, L, dev);
+}
+
 // fraction of a segment-row's lanes doing valid columns
 inline double lane_use(int Wo, int span) { return double(Wo) / (double(ceil_div(Wo, span)) * span); }
 
@@ -734,28 +867,51 @@ int launch_multi(const float *in, int N, int C, int H, int W, const float *filt,
     if (mv == 92) return launch_multi2_v<K, FBD, 1, 32, GUARDS, PF, 2, true>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
     if (mv == 93) return launch_multi2_v<K, FBD, 1, 16, GUARDS, PF, 2, true>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
   }
+  // 8: the r02 default (k_conv2d_multi2: 4 columns per lane, K-slot ring, FB = 8 / 2 filters per warp).
+  if (mv == 8) {
+    // Tuned on B200 (tools/multi_variants.py): 16-lane segments (two images per warp) unless they waste
+    // clearly more lanes than whole-warp rows -- more column blocks take the vector fast path and the
+    // ragged edge is a smaller share.
+    const bool seg16 = N >= 2 && lane_use(Wo, 64) >= lane_use(Wo, 128) - 0.05;
+    // 8-lane segments (four images per warp, 32 columns each) for narrow layers: Table I's 8-26-column
+    // outputs use 25-81% of the lanes instead of 12-41% (tools/multi_band_sweep.py)
+    const bool seg8 = N >= 4 && Wo <= 32 && lane_use(Wo, 32) >= lane_use(Wo, 64) + 0.15;
+    // K = 4..7 (two filters per warp): paired FMA across the filter pair (row_step_multi_p2, FFMA2) --
+    // profiles/r02p_multi_p2.txt: configs[3] 42.6 vs 37.6 TFLOP/s, Table I K=5 layers +5-20%. K <= 3 (eight
+    // filters per warp) keeps the scalar FMAs: its FFMA2 form spills at 3 CTAs per SM and loses at 2.
+    constexpr bool P2 = (K >= 4 && K <= 7 && FBD % 2 == 0);
+  #define C2D_LMP(SEGG) \
+    launch_multi2_v<K, FBD, 1, SEGG, GUARDS, PF, (SEGG == kWarp && K <= 3 && FBD >= 8) ? 2 : 3, P2>( \
+        in, N, C, H, W, filt, F, out, stream, band_h, dev)
+    if (seg8)
+      rc = C2D_LMP(8);
+    else
+      rc = seg16 ? C2D_LMP(16) : C2D_LMP(32);
+  #undef C2D_LMP
+    if (rc != CONV2D_ESHAPE) return rc;
+  }
 #undef C2D_LM2
+  // filter-blocked kernel (conv2d_mob.cuh) at a fixed shape: 100 FB=8 (3 CTAs per SM, K <= 8) / 101 FB=4
+  // with the automatic segment width; 102-105 FB=8 at 4/8/16/32-lane segments, 106-109 FB=4;
+  // 112 FB=8 with the L1 prefetch two rows ahead (K <= 8)
+  if (mv >= 100 && mv <= 112) {
+    constexpr int M4 = (K <= 6) ? 4 : 3;
+    const int segs[4] = {4, 8, 16, 32};
+    if (mv == 101) return launch_mob<K, 4, M4>(in, N, C, H, W, filt, F, out, stream, 0, 0, dev);
+    if (mv >= 106 && mv <= 109)
+      return launch_mob<K, 4, M4>(in, N, C, H, W, filt, F, out, stream, segs[mv - 106], 0, dev);
+    if constexpr (K <= 8) {
+      if (mv == 100) return launch_mob<K, 8, 3>(in, N, C, H, W, filt, F, out, stream, 0, 0, dev);
+      if (mv >= 102 && mv <= 105)
+        return launch_mob<K, 8, 3>(in, N, C, H, W, filt, F, out, stream, segs[mv - 102], 0, dev);
+      if (mv == 112) return launch_mob<K, 8, 3, true>(in, N, C, H, W, filt, F, out, stream, 0, 0, dev);
+    }
+    return CONV2D_EK;
+  }
 #endif
-  // Tuned on B200 (tools/multi_variants.py): 16-lane segments (two images per warp) unless they waste
-  // clearly more lanes than whole-warp rows -- more column blocks take the vector fast path and the
-  // ragged edge is a smaller share.
-  const bool seg16 = mv == 0 && N >= 2 && lane_use(Wo, 64) >= lane_use(Wo, 128) - 0.05;
-  // 8-lane segments (four images per warp, 32 columns each) for narrow layers: Table I's 8-26-column
-  // outputs use 25-81% of the lanes instead of 12-41% (tools/multi_band_sweep.py)
-  const bool seg8 = mv == 0 && N >= 4 && Wo <= 32 && lane_use(Wo, 32) >= lane_use(Wo, 64) + 0.15;
-  // K = 4..7 (two filters per warp): paired FMA across the filter pair (row_step_multi_p2, FFMA2) --
-  // profiles/r02p_multi_p2.txt: configs[3] 42.6 vs 37.6 TFLOP/s, Table I K=5 layers +5-20%. K <= 3 (eight
-  // filters per warp) keeps the scalar FMAs: its FFMA2 form spills at 3 CTAs per SM and loses at 2.
-  constexpr bool P2 = (K >= 4 && K <= 7 && FBD % 2 == 0);
-#define C2D_LMP(SEGG) \
-  launch_multi2_v<K, FBD, 1, SEGG, GUARDS, PF, (SEGG == kWarp && K <= 3 && FBD >= 8) ? 2 : 3, P2>( \
-      in, N, C, H, W, filt, F, out, stream, band_h, dev)
-  if (seg8)
-    rc = C2D_LMP(8);
-  else
-    rc = seg16 ? C2D_LMP(16) : C2D_LMP(32);
-#undef C2D_LMP
 #undef C2D_LM
+  // the filter-blocked kernel (conv2d_mob.cuh): profiles/r02_mob*, DESIGN.md section 5
+  rc = launch_mob_auto<K>(in, N, C, H, W, filt, F, out, stream, band_h, dev);
   if (rc != CONV2D_ESHAPE) return rc;
   // F-block does not fit shared memory: round-1 kernel with one filter per warp
   const size_t smem1 = static_cast<size_t>(C) * K * KP * sizeof(float);

@@ -21,6 +21,12 @@ ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 sys.path.insert(0, os.path.join(ROOT, "tools"))
 import ncu_raw_summary  # noqa: E402
 
+def dram_bytes(v: str) -> float:
+    """'1.502640 Gbyte' -> bytes (each metric carries its own unit)."""
+    num, unit = v.split()[:2]
+    return float(num.replace(",", "")) * {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9}[unit]
+
+
 # ncu capture name -> bench point name (tools/gpu_round.sh profiles these configurations)
 CAPTURES = {
     "prof_k15_b8_s8192": "conv2d_single 8192^2 K=15 x8 images",
@@ -101,11 +107,7 @@ def main():
             fh.write(f"# ncu --set full --clock-control none, {point}\n")
             for k, v in s.items():
                 fh.write(f"{k}: {v}\n")
-        rd = float(s["dram__bytes_read.sum"].split()[0].replace(",", ""))
-        wr = float(s["dram__bytes_write.sum"].split()[0].replace(",", ""))
-        unit = s["dram__bytes_read.sum"].split()[1]
-        scale = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9}[unit]
-        traffic[point] = round((rd + wr) * scale)
+        traffic[point] = round(dram_bytes(s["dram__bytes_read.sum"]) + dram_bytes(s["dram__bytes_write.sum"]))
     json.dump(traffic, open(traffic_path, "w"), indent=1)
     print("profiles written:", sorted(os.listdir(dst)))
 
