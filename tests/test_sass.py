@@ -4,7 +4,7 @@ The paper's dynamic->static index transformation exists to 
 window (iTemp) and the output accumulators (Out) in registers: a kernel that spills them to local
 memory has lost exactly what the method is about. Every kernel shipped in libconv2d.so must therefore
 be free of LDL/STL, and the single-channel kernels must show the method's instruction signature:
-FFMA for row reuse and SHFL for column reuse."""
+FFMA / FFMA2 for row reuse and SHFL for column reuse; the multi-channel kernels FFMA2 over filter pairs."""
 import os
 import sys
 
@@ -33,7 +33,7 @@ def test_single_channel_kernels_carry_column_and_row_reuse(product_kernels):
     singles = {k: c for k, c in product_kernels.items() if "k_conv2d_single" in k or "k_conv2d_split" in k}
     assert singles
     for k, c in singles.items():
-        assert c["FFMA"] > 0, k
+        assert c["FFMA"] + c["FFMA2"] > 0, k  # row reuse: FMA chains (scalar, or paired fma.rn.f32x2)
         kk = int(k.split("ILi", 1)[1].split("E", 1)[0])  # K, the first template argument
         if kk > 1:
             assert c["SHFL"] > 0, k  # column reuse: halo columns by warp shuffle, not reloads
@@ -44,3 +44,15 @@ def test_tensor_core_variant_uses_tcgen05(product_kernels):
     assert tc
     for k, c in tc.items():
         assert c["UTCHMMA"] + c["UTCQMMA"] > 0 and c["LDTM"] > 0, k
+
+
+def test_multi_channel_kernels_pair_filters_and_shuffle(product_kernels):
+    """The filter-blocked multi-channel kernel (conv2d_mob.cuh): paired FMAs over filter pairs, broadcast
+    LDS of the staged F-block, SHFL for the column-reuse halo (K > 1)."""
+    mob = {k: c for k, c in product_kernels.items() if "k_conv2d_mob" in k}
+    assert mob
+    for k, c in mob.items():
+        assert c["FFMA2"] > 0 and c["LDS"] > 0, k
+        kk = int(k.split("ILi", 1)[1].split("E", 1)[0])
+        if kk > 1:
+            assert c["SHFL"] > 0, k

@@ -20,7 +20,7 @@ import sys
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 PKG = os.path.join(ROOT, "paper_conf_cluster_luzw20_b200")
 LIBS = {"product": os.path.join(PKG, "libconv2d.so"), "tune": os.path.join(PKG, "libconv2d_tune.so")}
-COLS = ["FFMA", "SHFL", "FSEL", "SEL", "LDCU", "LDC", "LDS", "LDG", "LDGSTS", "STG", "STS", "LDL", "STL",
+COLS = ["FFMA", "FFMA2", "SHFL", "FSEL", "SEL", "LDCU", "LDC", "LDS", "LDG", "LDGSTS", "STG", "STS", "LDL", "STL",
         "UTCHMMA", "UTCQMMA", "LDTM", "STTM", "UBLKCP", "BAR", "SYNCS"]
 
 
