@@ -45,8 +45,8 @@ prof prof_k15_s4096 "k_conv2d_(single|wide)" single 4096 15
 prof prof_k5_s2048 "k_conv2d_(single|wide)" single 2048 5
 prof prof_direct_k3_s8192 k_conv2d_direct single 8192 3 --direct
 prof prof_split_k15_s1024 k_conv2d_split single 1024 15
-prof prof_conv11c1 k_conv2d_multi multi 128,1,224,224,64 3
-prof prof_multi_config3 k_conv2d_multi multi 128,3,224,224,64 7
+prof prof_conv11c1 "k_conv2d_(mob|multi2)" multi 128,1,224,224,64 3
+prof prof_multi_config3 "k_conv2d_(mob|multi2)" multi 128,3,224,224,64 7
 prof prof_tc_config2 k_conv2d_multi_tc multi 32,64,56,56,64 3 --tc
 prof prof_tc_config3 k_conv2d_multi_tc multi 128,3,224,224,64 7 --tc
 prof prof_config0 "k_conv2d_(single|wide)" single 256 3
