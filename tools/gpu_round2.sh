@@ -38,9 +38,9 @@ prof() {  # name, kernel regex, prof_one.py args
   ncu -i /tmp/$n.ncu-rep --page source --csv --print-source sass > gpurun_out/$n.src.csv 2>/dev/null
   gzip -f gpurun_out/$n.src.csv
 }
-prof prof_k15_b8_s8192 "k_conv2d_(single|wide)" single 8192 15 --batch 8
+prof prof_k15_b8_s8192 "k_conv2d_(single|wide|pair)" single 8192 15 --batch 8
 prof prof_k3_b8_s8192 "k_conv2d_(single|wide)" single 8192 3 --batch 8
-prof prof_k7_b8_s8192 "k_conv2d_(single|wide)" single 8192 7 --batch 8
+prof prof_k7_b8_s8192 "k_conv2d_(single|wide|pair)" single 8192 7 --batch 8
 prof prof_k15_s4096 "k_conv2d_(single|wide)" single 4096 15
 prof prof_k5_s2048 "k_conv2d_(single|wide)" single 2048 5
 prof prof_direct_k3_s8192 k_conv2d_direct single 8192 3 --direct
