@@ -665,7 +665,8 @@ def _run_e2e(points, unit, args, device):
     import paper_conf_cluster_luzw20_b200 as pkg
 
     main = torch.cuda.current_stream(device)
-    streams = [torch.cuda.Stream(device=device) for _ in range(2)]
+    ns = max(1, args.e2e_streams)
+    streams = [torch.cuda.Stream(device=device) for _ in range(ns)]
     # host buffers: one pinned input / output per distinct shape (the host side has no L2 to defeat)
     hx, hy = {}, {}
     for p in points:
@@ -687,10 +688,10 @@ def _run_e2e(points, unit, args, device):
             if p.kind == "single":
                 xin, yout = hx[(p.dims, p.n_local)], hy[key]
                 for j in range(p.n_local):
-                    pkg.conv2d_single_host(xin[j], hf[i], device=device, stream=streams[c % 2], out_host=yout[j])
+                    pkg.conv2d_single_host(xin[j], hf[i], device=device, stream=streams[c % ns], out_host=yout[j])
                     c += 1
             else:
-                pkg.conv2d_multi_host(hx[key], hf[i], device=device, stream=streams[c % 2], out_host=hy[key],
+                pkg.conv2d_multi_host(hx[key], hf[i], device=device, stream=streams[c % ns], out_host=hy[key],
                                       impl=args.multi_impl)
                 c += 1
         for s in streams:
@@ -711,9 +712,9 @@ def _run_e2e(points, unit, args, device):
     d2h = sum(4 * p.y.numel() for p in points)
     return {"value": round(units / (ms * 1e-3) / 1e9, 3), "unit": unit, "h2d_bytes_per_step": h2d,
             "d2h_bytes_per_step": d2h, "steps": steps, "ms_per_step": round(ms / steps, 3),
-            "path": ("conv2d_single_host (C ABI, pinned host buffers, one call per image, 2 streams)"
+            "path": (f"conv2d_single_host (C ABI, pinned host buffers, one call per image, {ns} streams)"
                      if points[0].kind == "single" else
-                     f"conv2d_multi_host (impl={args.multi_impl}; pinned host buffers, 2 streams)")}
+                     f"conv2d_multi_host (impl={args.multi_impl}; pinned host buffers, {ns} streams)")}
 
 
 def load_traffic(kernel_name):
@@ -859,6 +860,7 @@ def main():
                     help=f"images per single-channel point (sweep default {DEFAULT_SWEEP_BATCH}, config0 default 1); "
                          "split across ranks")
     ap.add_argument("--e2e-steps", type=int, default=3)
+    ap.add_argument("--e2e-streams", type=int, default=2, help="e2e: caller streams the per-image host calls alternate over")
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--cpu-budget", type=float, default=10.0)
