@@ -153,6 +153,14 @@ __global__ void __launch_bounds__(kCtaWarps *kWarp, MINB) k_conv2d_mob(const Mob
     nx0 = fx0;
     if (nsteps > 1) unit_of(s0 + kCtaWarps, nrp, nx0, oi, vd);
   }
+  // the fetch row's 64-bit base formed once per row (opaque to the compiler, which otherwise folds the
+  // row offset into every quad's column offset and redoes the 64-bit scaling per load)
+  // (K >= 5: configs[3] 49.7 -> 50.8 TFLOP/s; at K <= 4 it costs the L1-prefetch form its last registers)
+  auto row_ptr = [&](int off) {
+    const float *p = a.in + off;
+    if constexpr (K >= 5) asm("" : "+l"(p));
+    return p;
+  };
   const int wrap = a.W - (C - 1) * plane;  // (i, C-1) -> (i+1, 0); |wrap| < 2^31 (checked by the launcher)
   auto advance = [&]() {
     const bool cw = fc + 1 < C;
@@ -198,7 +206,7 @@ __global__ void __launch_bounds__(kCtaWarps *kWarp, MINB) k_conv2d_mob(const Mob
     fa += fstride;
   };
   WideRow bufA, bufB;
-  wide_load<K, EDGE, SEG>(bufA, a.in + frow, fx0, a.W, sl);
+  wide_load<K, EDGE, SEG>(bufA, row_ptr(frow), fx0, a.W, sl);
   advance();
   // one warp-step starting from buffer X (rows t, t+1 in pairs; an odd last row leaves the next
   // step's row 0 in the other buffer)
@@ -206,15 +214,15 @@ __global__ void __launch_bounds__(kCtaWarps *kWarp, MINB) k_conv2d_mob(const Mob
     int t = 0;
 #pragma unroll 1
     for (; t + 1 < rows; t += 2) {
-      wide_load<K, EDGE, SEG>(Y, a.in + frow, fx0, a.W, sl);
+      wide_load<K, EDGE, SEG>(Y, row_ptr(frow), fx0, a.W, sl);
       advance();
       compute(X);
-      wide_load<K, EDGE, SEG>(X, a.in + frow, fx0, a.W, sl);
+      wide_load<K, EDGE, SEG>(X, row_ptr(frow), fx0, a.W, sl);
       advance();
       compute(Y);
     }
     if (t < rows) {
-      wide_load<K, EDGE, SEG>(Y, a.in + frow, fx0, a.W, sl);
+      wide_load<K, EDGE, SEG>(Y, row_ptr(frow), fx0, a.W, sl);
       advance();
       compute(X);
     }
