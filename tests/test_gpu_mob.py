@@ -105,3 +105,42 @@ def test_small_grid_takes_fb4(cuda_device):
     finally:
         _capi.debug_set_multi_variant(0)
     assert torch.equal(y, y8)
+
+
+def test_cuda_graph_capture_and_concurrent_streams(cuda_device):
+    """conv2d_multi captured into a CUDA graph replays correctly and picks up new inputs and filters at
+    replay; calls with different filters on three streams give the one-stream bits (the F-block is
+    staged per CTA from the caller's filter tensor: no library-global state between calls)."""
+    x = dev_image((6, 3, 60, 90), "img", seed=3)
+    w = _w(20, 3, 5, seed=3)
+    y = torch.empty((6, 20, 56, 86), device=DEV)
+    s = torch.cuda.Stream()
+    s.wait_stream(torch.cuda.current_stream())
+    with torch.cuda.stream(s):
+        pkg.conv2d_multi(x, w, out=y)  # warm-up outside capture (occupancy and smem attributes)
+    torch.cuda.current_stream().wait_stream(s)
+    g = torch.cuda.CUDAGraph()
+    with torch.cuda.graph(g):
+        pkg.conv2d_multi(x, w, out=y)
+    g.replay()
+    torch.cuda.synchronize()
+    check_full_multi(x, w, y)
+    x.copy_(dev_image((6, 3, 60, 90), "sym", seed=4))
+    w.copy_(_w(20, 3, 5, seed=4))
+    g.replay()
+    torch.cuda.synchronize()
+    check_full_multi(x, w, y)
+
+    ws = [_w(12, 3, 7, seed=10 + i) for i in range(6)]
+    xs = dev_image((4, 3, 40, 230), "img", seed=11)
+    outs = [torch.empty((4, 12, 34, 224), device=DEV) for _ in ws]
+    streams = [torch.cuda.Stream() for _ in range(3)]
+    for st in streams:
+        st.wait_stream(torch.cuda.current_stream())
+    for i, wi in enumerate(ws):
+        st = streams[i % 3]
+        with torch.cuda.stream(st):
+            pkg.conv2d_multi(xs, wi, out=outs[i], stream=st)
+    torch.cuda.synchronize()
+    for wi, yi in zip(ws, outs):
+        assert torch.equal(yi, pkg.conv2d_multi(xs, wi))
