@@ -144,3 +144,14 @@ def test_cuda_graph_capture_and_concurrent_streams(cuda_device):
     torch.cuda.synchronize()
     for wi, yi in zip(ws, outs):
         assert torch.equal(yi, pkg.conv2d_multi(xs, wi))
+
+
+@pytest.mark.parametrize("C,K", [(40, 15), (200, 15), (300, 9)])
+def test_large_c_fallback(cuda_device, C, K):
+    """F-blocks beyond shared memory: C*K*K*8*4 B (FB = 8) or *4 (FB = 4) past the opt-in limit hand over
+    to FB = 4 or to the round-1 kernel with one filter per warp (C*K*ceil(K/4)*16 B); every output
+    against the oracle either way."""
+    x = dev_image((1, C, K + 3, K + 40), "sym", seed=C)
+    w = _w(5, C, K, seed=C)
+    y = pkg.conv2d_multi(x, w)
+    check_full_multi(x, w, y)
