@@ -792,17 +792,17 @@ int launch_mob(const float *in, int N, int C, int H, int W, const float *filt, i
 }
 
 // The product multi-channel path (conv2d_mob.cuh). FB = 8 filters per lane at 3 CTAs per SM (168
-// registers) for K <= 8 except K = 5, unless its grid fills less than 3/4 of one wave -- then FB = 4
-// (twice the CTAs, 4 CTAs per SM up to K = 6): Table I CONV4/6/7, tools/multi_variants.py,
-// profiles/r02_mob*. K = 5 and K >= 9: FB = 4 (ptxas spills FB = 8 there at 168 registers; 0 LDL/STL
-// in every product kernel, tests/test_sass.py). band_h > 0: warp-steps per warp (explicit tiling;
-// same bits). Returns CONV2D_ESHAPE when the F-block does not fit shared memory (caller falls back).
+// registers) for K <= 8, unless its grid fills less than 3/4 of one wave -- then FB = 4 (twice the
+// CTAs, 4 CTAs per SM up to K = 6): Table I CONV4/6/7, tools/multi_variants.py, profiles/r02mob*.
+// K >= 9: FB = 4 (ptxas spills FB = 8 there at 168 registers; 0 LDL/STL in every product kernel,
+// tests/test_sass.py). band_h > 0: warp-steps per warp (explicit tiling; same bits). Returns
+// CONV2D_ESHAPE when the F-block does not fit shared memory (caller falls back).
 template <int K>
 int launch_mob_auto(const float *in, int N, int C, int H, int W, const float *filt, int F, float *out,
                     cudaStream_t stream, int band_h, const DevInfo &dev) {
   constexpr int M4 = (K <= 6) ? 4 : 3;
   const int L = band_h > 0 ? band_h : 0;
-  if constexpr (K <= 8 && K != 5) {
+  if constexpr (K <= 8) {
     long long plan[2] = {0, 0};
     const int e = launch_mob<K, 8, 3>(in, N, C, H, W, filt, F, out, stream, 0, L, dev, plan);
     if (e == CONV2D_OK && 4 * plan[0] >= 3 * plan[1]) {
