@@ -2,8 +2,8 @@
 """Small invocations of every product kernel family for compute-sanitizer (memcheck / racecheck /
 initcheck): wide-lane and one-chunk single-channel kernels (register and cp.async-ring row fetch, shared
 and constant filters), the filter-row split kernel (cluster of 2 CTAs, DSMEM), batches, the halo and
-'same'-padding paths, rectangular filters, the multi-channel kernel (cp.async ring, 8/16/32-lane
-segments, misaligned input) and the tcgen05 tensor-core variant, the host-buffer pipeline.
+'same'-padding paths, rectangular filters, the multi-channel kernels (filter-blocked default at 4/8/16-lane
+segments, FB = 8 / 4, misaligned input, large-C fallbacks) and the tcgen05 tensor-core variant, the host-buffer pipeline.
 
     compute-sanitizer --tool memcheck python tools/sanitize_cases.py
 """
@@ -38,8 +38,12 @@ def main():
         pkg.conv2d_single_halo(img((40, 600)), img((K - 1, 600), 3), filt(K))
         pkg.conv2d_single_pad(img((50, 260)), filt(K), "same_replicate", flip=True)
         pkg.conv2d_single_rect(img((K + 30, 530)), torch.rand((K, max(1, K - 2)), device="cuda"))
+    # multi-channel: the filter-blocked kernel at 4/8/16-lane segments, FB = 8 and 4, the K <= 4 L1-prefetch
+    # form, odd output pitch, the large-C fallbacks (FB = 4, then the one-filter round-1 kernel)
     for (N, C, H, W, F, K) in [(4, 3, 30, 33, 16, 3), (2, 64, 20, 20, 64, 3), (1, 3, 40, 260, 8, 7),
-                               (5, 1, 28, 28, 20, 5), (2, 2, 19, 23, 3, 15)]:
+                               (5, 1, 28, 28, 20, 5), (2, 2, 19, 23, 3, 15), (3, 3, 20, 224, 24, 7),
+                               (4, 8, 14, 56, 16, 3), (2, 3, 12, 29, 9, 5), (1, 40, 20, 60, 5, 15),
+                               (1, 200, 18, 40, 3, 15)]:
         x = img((N, C, H, W))
         w = torch.from_numpy(synth.make_filter(4, K, "he", F=F, C=C)).cuda()
         pkg.conv2d_multi(x, w)
