@@ -47,7 +47,8 @@ def main():
         x = img((N, C, H, W))
         w = torch.from_numpy(synth.make_filter(4, K, "he", F=F, C=C)).cuda()
         pkg.conv2d_multi(x, w)
-        pkg.conv2d_multi_tc(x, w)
+        if C * K * K <= (1 << 14):  # the tensor-core variant's im2col offset table bound (conv2d.h)
+            pkg.conv2d_multi_tc(x, w)
         xb = img((N * C * H * W + 1,))[1:].view(N, C, H, W)  # misaligned input
         pkg.conv2d_multi(xb, w)
     xh = torch.rand((70, 300)).pin_memory()
