@@ -1,5 +1,13 @@
+#!/usr/bin/env python
+"""'same'-padding call (conv2d_single_pad) vs the valid call at 8192^2 K = 3/5/7 across single-channel
+kernel variants (tuning build): us per call, bits checked across variants.
+
+    python tools/pad_variants.py
+"""
 import sys, torch
-sys.path.insert(0, '/root/repo'); sys.path.insert(0, '/root/repo/tools')
+import os
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT); sys.path.insert(0, os.path.join(ROOT, 'tools'))
 import paper_conf_cluster_luzw20_b200 as pkg
 from paper_conf_cluster_luzw20_b200 import _capi
 from gen import synth
