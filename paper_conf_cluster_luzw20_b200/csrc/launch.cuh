@@ -725,12 +725,21 @@ int launch_mob_k(const float *in, int N, int C, int H, int W, const float *filt,
   const long long resident =
       static_cast<long long>(cta_occupancy(kernel, smem, occ_cache, kCtaWarps * kWarp)) * dev.num_sms;
   if (L <= 0) {
+    // Only the smallest L of each wave count can be optimal (cost grows with L at fixed waves): for
+    // w = 1 .. waves(L = 1), L_w = the smallest L whose grid fits in w waves. O(waves) host work per
+    // call instead of O(steps); scanned with L ascending so ties keep the smallest L.
     const long long lmax = (a.steps + kCtaWarps - 1) / kCtaWarps;
+    auto ctas_of = [&](long long l) { return static_cast<long long>(n_fb) * ((a.steps + kCtaWarps * l - 1) / (kCtaWarps * l)); };
+    const long long w1 = (ctas_of(1) + resident - 1) / resident;
     double best = 1e300;
     L = 1;
-    for (long long l = 1; l <= lmax; ++l) {
-      const long long ctas = static_cast<long long>(n_fb) * ((a.steps + kCtaWarps * l - 1) / (kCtaWarps * l));
-      const long long waves = (ctas + resident - 1) / resident;
+    for (long long w = w1 < 65536 ? w1 : 65536; w >= 1; --w) {
+      const long long m = w * resident / n_fb;  // CTAs per F-block that fit in w waves
+      if (m < 1) continue;
+      long long l = (a.steps + kCtaWarps * m - 1) / (kCtaWarps * m);
+      if (l < 1) l = 1;
+      if (l > lmax) l = lmax;
+      const long long waves = (ctas_of(l) + resident - 1) / resident;
       const double cost = static_cast<double>(waves) * (static_cast<double>(l) + 0.05);
       if (cost < best - 1e-9) {
         best = cost;
